@@ -1,0 +1,164 @@
+/*
+ * lift.h — C ABI of the B200-native Lift hot path:
+ *          the fused zip -> map(x) -> reduce(+) kernel with no intermediate
+ *          arrays, instantiated for dot, GEMV, GESUMMV and ATAX.
+ *
+ * Citations are PAPER.md line numbers (L<n>) of Steuwer, Remmelg, Dubach,
+ * "Lift: A Functional Data-Parallel IR for High-Performance GPU Code
+ * Generation", CGO 2017 (the file /root/reference/PAPER.md of the build).
+ *
+ * Conventions shared by every entry point
+ * ---------------------------------------
+ *  - Data: fp32 ("All experiments are performed using single precision
+ *    floats", L1003).  Matrices are dense, row-major, contiguous, lda = n
+ *    (reading R10).  Sizes are int64 (2^31-element configs; Fig. 7
+ *    uses `int N`, L950 — widened, reading R7).
+ *  - Pointers: every array pointer is a DEVICE pointer on the calling
+ *    thread's current CUDA device, at least 4-byte aligned.  16-byte aligned
+ *    bases with n % 4 == 0 take the 128-bit vector path (asVector4, L378-389);
+ *    anything else takes the scalar path (same results contract).
+ *  - Ownership: the caller owns every buffer.  The library never allocates,
+ *    frees, synchronises, or changes the current device.
+ *  - Streams: `stream` is a cudaStream_t (NULL = legacy default stream).
+ *    Work is enqueued asynchronously; calls are CUDA-graph capturable.
+ *  - restrict: outputs must not overlap inputs or the workspace (Fig. 7
+ *    declares `restrict` inputs, L948-950); overlap -> LIFT_ERR_ALIAS.
+ *  - Errors: argument validation happens on the host BEFORE anything touches
+ *    CUDA and returns a status with nothing enqueued.  LIFT_ERR_CUDA reports a
+ *    launch/configuration error (text via lift_last_cuda_error()).  Faults
+ *    during execution surface at the caller's next stream synchronisation.
+ *  - Determinism: no floating-point atomics; for a fixed (shape, device) the
+ *    output is bitwise reproducible.  GEMV/GESUMMV rows use one canonical
+ *    summation order that depends only on n, so row-sharded results are
+ *    bitwise equal to unsharded ones.
+ *  - Accuracy contract (BASELINE.json north_star): elementwise
+ *    |out - exact| <= 1e-5 * sum|terms| + 1e-6, fp32 accumulation in FMA.
+ *  - Empty sizes: n == 0 -> dot writes 0, GEMV family writes y = 0 (m rows);
+ *    m == 0 -> GEMV family is a no-op, ATAX writes y = 0 (n entries).
+ */
+#ifndef LIFT_H
+#define LIFT_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#if defined(__GNUC__)
+#define LIFT_API __attribute__((visibility("default")))
+#else
+#define LIFT_API
+#endif
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+/* Same type as cudaStream_t, without requiring CUDA headers. */
+typedef struct CUstream_st *lift_stream_t;
+
+typedef enum lift_status {
+    LIFT_OK = 0,
+    LIFT_ERR_NULL_PTR = 1,   /* a pointer needed for a non-empty size is NULL          */
+    LIFT_ERR_BAD_SIZE = 2,   /* negative size, m*n overflows int64, or size rule broken */
+    LIFT_ERR_MISALIGNED = 3, /* a pointer is not 4-byte aligned                        */
+    LIFT_ERR_ALIAS = 4,      /* an output range overlaps an input / workspace range    */
+    LIFT_ERR_WORKSPACE = 5,  /* workspace NULL, too small, or not 16-byte aligned      */
+    LIFT_ERR_CUDA = 6        /* CUDA launch / attribute error (lift_last_cuda_error()) */
+} lift_status;
+
+/* ---------------------------------------------------------------------- */
+/* dot:  *result = sum_i x_i * y_i                                         */
+/* ---------------------------------------------------------------------- */
+/* dot(x, y) = reduce(+, 0, map(x, zip(x, y)))  — L285, Sec. 3.1; lowered as
+ * Listing 1 (L391-401): per-thread reduceSeq(multAndSumUp, 0) over a chunk
+ * (L398-399), an in-block tree (iterate6, L394-397) and a second stage over
+ * the per-block results (L422-426) — here fused into ONE launch (the last
+ * block to finish reduces the partials in a fixed order).
+ *
+ *   n          number of elements (>= 0)
+ *   x, y       device fp32[n]
+ *   result     device fp32[1], written (never read)
+ *   workspace  device scratch of >= lift_dot_workspace_bytes(n) bytes,
+ *              16-byte aligned.  Its first 16 bytes hold an arrival ticket
+ *              that MUST be zero before the first call (e.g. cudaMemset once
+ *              at allocation); every call leaves it zero again.  One
+ *              workspace must not be used by concurrent calls.           */
+LIFT_API size_t lift_dot_workspace_bytes(int64_t n);
+LIFT_API int lift_dot(int64_t n, const float *x, const float *y, float *result,
+             void *workspace, size_t workspace_bytes, lift_stream_t stream);
+
+/* ---------------------------------------------------------------------- */
+/* GEMV:  y = A x                                                          */
+/* ---------------------------------------------------------------------- */
+/* Table 1 GEMV (L1030; CLBlast, 4K^2 / 8K^2).  y_i is dot(A_i, x): rows are
+ * distributed over blocks (mapWrg, L359-367) and x is staged once per block
+ * in shared memory (toLocal, L368-377) by the bulk-copy (TMA) engine.
+ * Reading R8: y = A x, y written and never read (BLAS alpha = 1, beta = 0).
+ *
+ *   m, n   rows, columns (>= 0)
+ *   A      device fp32[m][n] row-major
+ *   x      device fp32[n]
+ *   y      device fp32[m], written                                       */
+LIFT_API int lift_gemv(int64_t m, int64_t n, const float *A, const float *x, float *y,
+              lift_stream_t stream);
+
+/* ---------------------------------------------------------------------- */
+/* GESUMMV:  y = alpha A x + beta B x                                      */
+/* ---------------------------------------------------------------------- */
+/* Table 1 GESUMMV (L1031).  Reading R9 (PolyBench): y = alpha*Ax + beta*Bx.
+ * One kernel streams the zipped rows (A_i, B_i) (zip, L343-347) with two
+ * accumulators; neither A x nor B x is materialised.  Epilogue per row:
+ * y_i = alpha*sA + beta*sB, each product rounded, then one rounded add.
+ *
+ *   alpha, beta  fp32 scalars (by value)
+ *   A, B         device fp32[m][n] row-major
+ *   x            device fp32[n];  y device fp32[m], written              */
+LIFT_API int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, float beta,
+                 const float *B, const float *x, float *y, lift_stream_t stream);
+
+/* ---------------------------------------------------------------------- */
+/* ATAX:  y = A^T (A x)                                                    */
+/* ---------------------------------------------------------------------- */
+/* Table 1 ATAX (L1029).  Reading R9: t = A x (t in R^m, fp32), y = A^T t
+ * (y in R^n).  The transpose is never materialised: A^T is read through the
+ * transposed index l_id*N + wg_id (Fig. 6; matrixTranspose
+ * L848-850).
+ *
+ * lift_atax picks the fastest algorithm for the shape:
+ *   LIFT_ATAX_FUSED    one streaming pass over A: per row group, t_r = A_r x
+ *                      by a block tree, then y_part += A_r^T t_r from the
+ *                      same registers; then a fixed-order reduce of the
+ *                      per-block y_part (reads A once: 4*m*n bytes).
+ *   LIFT_ATAX_TWOPASS  the paper's structure (two GEMV-shaped kernels whose
+ *                      times are summed, L1006-1007): GEMV t = A x, then a
+ *                      column-blocked A^T t into per-row-split partials, then
+ *                      a fixed-order reduce (reads A twice: 8*m*n bytes).
+ *
+ *   A          device fp32[m][n] row-major;  x device fp32[n]
+ *   y          device fp32[n], written
+ *   workspace  device scratch >= lift_atax_workspace_bytes(m, n), 16-byte
+ *              aligned; no initialisation needed; not shared by concurrent
+ *              calls.                                                     */
+typedef enum lift_atax_algo {
+    LIFT_ATAX_AUTO = 0,
+    LIFT_ATAX_FUSED = 1,
+    LIFT_ATAX_TWOPASS = 2
+} lift_atax_algo;
+
+LIFT_API size_t lift_atax_workspace_bytes(int64_t m, int64_t n);
+LIFT_API int lift_atax(int64_t m, int64_t n, const float *A, const float *x, float *y,
+              void *workspace, size_t workspace_bytes, lift_stream_t stream);
+LIFT_API int lift_atax_algo_run(int algo, int64_t m, int64_t n, const float *A,
+                       const float *x, float *y, void *workspace,
+                       size_t workspace_bytes, lift_stream_t stream);
+
+/* ---------------------------------------------------------------------- */
+/* library info                                                            */
+/* ---------------------------------------------------------------------- */
+LIFT_API const char *lift_strerror(int status);      /* static string, never NULL   */
+LIFT_API const char *lift_last_cuda_error(void);     /* thread-local, last CUDA error text */
+LIFT_API int lift_version(void);                     /* (major << 16) | minor        */
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* LIFT_H */

@@ -1,0 +1,173 @@
+"""B200-native Lift hot path: the fused zip -> map(x) -> reduce(+) kernel
+(Steuwer, Remmelg, Dubach, CGO 2017) for dot, GEMV, GESUMMV and ATAX.
+
+Thin Python binding over the C ABI in ``include/lift.h`` (``liblift.so``):
+every step of the path runs in the library's CUDA kernels; this module only
+checks tensors, allocates outputs / workspaces with torch, and passes raw
+device pointers plus ``torch.cuda.current_stream()``.  The function names are
+the C names.  Inputs must be fp32, contiguous CUDA tensors on one device.
+
+Sharded (multi-GPU) variants live in :mod:`paper_conf_cgo_steuwerrd17_b200.shard`.
+"""
+from __future__ import annotations
+
+import threading
+
+import torch
+
+from ._lib import (LIFT_ATAX_AUTO, LIFT_ATAX_FUSED, LIFT_ATAX_TWOPASS, LiftError,  # noqa: F401
+                   check, lib, library_path)
+
+__all__ = ["lift_dot", "lift_gemv", "lift_gesummv", "lift_atax", "lift_gemv_tuned", "lift_gesummv_tuned",
+           "LiftError", "lib", "library_path", "KERNELS_PER_CALL"]
+
+# kernels each entry point enqueues (for the bench's gpu_launches count)
+KERNELS_PER_CALL = {"lift_dot": 1, "lift_gemv": 1, "lift_gesummv": 1, "lift_atax_fused": 2, "lift_atax_twopass": 3}
+
+_ws_lock = threading.Lock()
+_ws_cache: dict = {}
+
+
+def _check_tensor(t: torch.Tensor, name: str, dim: int | None = None) -> None:
+    if not isinstance(t, torch.Tensor):
+        raise TypeError(f"{name} must be a torch.Tensor")
+    if t.dtype != torch.float32:
+        raise TypeError(f"{name} must be float32 (got {t.dtype})")
+    if t.device.type != "cuda":
+        raise ValueError(f"{name} must be a CUDA tensor (got {t.device}); there is no CPU path")
+    if not t.is_contiguous():
+        raise ValueError(f"{name} must be contiguous")
+    if dim is not None and t.dim() != dim:
+        raise ValueError(f"{name} must be {dim}-D (got shape {tuple(t.shape)})")
+
+
+def _same_device(*ts: torch.Tensor) -> torch.device:
+    d = ts[0].device
+    for t in ts[1:]:
+        if t.device != d:
+            raise ValueError(f"tensors on different devices: {d} vs {t.device}")
+    return d
+
+
+def _stream(device: torch.device) -> int:
+    return torch.cuda.current_stream(device).cuda_stream
+
+
+def _workspace(kind: str, device: torch.device, nbytes: int, zero: bool) -> torch.Tensor:
+    """Per-(kind, device, stream) cached workspace, grown on demand.
+
+    The dot workspace holds an arrival ticket that must start at zero; it is
+    allocated with torch.zeros and every dot call leaves it zero again."""
+    key = (kind, device.index, _stream(device))
+    with _ws_lock:
+        ws = _ws_cache.get(key)
+        if ws is None or ws.numel() < nbytes:
+            alloc = torch.zeros if zero else torch.empty
+            ws = alloc(max(nbytes, 256), dtype=torch.uint8, device=device)
+            _ws_cache[key] = ws
+        return ws
+
+
+def lift_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None = None) -> torch.Tensor:
+    """0-d fp32 CUDA tensor sum_i x_i*y_i  (Listing 1)."""
+    _check_tensor(x, "x", 1)
+    _check_tensor(y, "y", 1)
+    dev = _same_device(x, y)
+    if x.numel() != y.numel():
+        raise ValueError("x and y must have the same length")
+    if out is None:
+        out = torch.empty((), dtype=torch.float32, device=dev)
+    _check_tensor(out, "out")
+    L = lib()
+    n = x.numel()
+    nbytes = L.lift_dot_workspace_bytes(n)
+    with torch.cuda.device(dev):
+        ws = _workspace("dot", dev, nbytes, zero=True)
+        check(L.lift_dot(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(), _stream(dev)))
+    return out
+
+
+def lift_gemv(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None) -> torch.Tensor:
+    """y = A x, A (m, n) row-major fp32  (Table 1 GEMV, L1030)."""
+    _check_tensor(A, "A", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, x)
+    m, n = A.shape
+    if x.numel() != n:
+        raise ValueError(f"x has {x.numel()} elements, A has {n} columns")
+    if out is None:
+        out = torch.empty(m, dtype=torch.float32, device=dev)
+    _check_tensor(out, "out", 1)
+    with torch.cuda.device(dev):
+        check(lib().lift_gemv(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), _stream(dev)))
+    return out
+
+
+def lift_gemv_tuned(A, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1):
+    """lift_gemv with an explicit launch configuration (include/lift_tuning.h)."""
+    _check_tensor(A, "A", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, x)
+    m, n = A.shape
+    if out is None:
+        out = torch.empty(m, dtype=torch.float32, device=dev)
+    with torch.cuda.device(dev):
+        check(lib().lift_gemv_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), wpr, rg, blocks, xsmem,
+                                    _stream(dev)))
+    return out
+
+
+def lift_gesummv(alpha: float, A: torch.Tensor, beta: float, B: torch.Tensor, x: torch.Tensor,
+                 out: torch.Tensor | None = None) -> torch.Tensor:
+    """y = alpha A x + beta B x  (Table 1 GESUMMV, L1031); alpha/beta passed as fp32."""
+    _check_tensor(A, "A", 2)
+    _check_tensor(B, "B", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, B, x)
+    m, n = A.shape
+    if tuple(B.shape) != (m, n) or x.numel() != n:
+        raise ValueError("shape mismatch")
+    if out is None:
+        out = torch.empty(m, dtype=torch.float32, device=dev)
+    _check_tensor(out, "out", 1)
+    with torch.cuda.device(dev):
+        check(lib().lift_gesummv(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
+                                 out.data_ptr(), _stream(dev)))
+    return out
+
+
+def lift_gesummv_tuned(alpha, A, beta, B, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1):
+    _check_tensor(A, "A", 2)
+    _check_tensor(B, "B", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, B, x)
+    m, n = A.shape
+    if out is None:
+        out = torch.empty(m, dtype=torch.float32, device=dev)
+    with torch.cuda.device(dev):
+        check(lib().lift_gesummv_tuned(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
+                                       out.data_ptr(), wpr, rg, blocks, xsmem, _stream(dev)))
+    return out
+
+
+_ALGOS = {"auto": LIFT_ATAX_AUTO, "fused": LIFT_ATAX_FUSED, "twopass": LIFT_ATAX_TWOPASS}
+
+
+def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None, algo: str = "auto") -> torch.Tensor:
+    """y = A^T (A x)  (Table 1 ATAX, L1029).  algo: "auto" | "fused" | "twopass"."""
+    _check_tensor(A, "A", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, x)
+    m, n = A.shape
+    if x.numel() != n:
+        raise ValueError(f"x has {x.numel()} elements, A has {n} columns")
+    if out is None:
+        out = torch.empty(n, dtype=torch.float32, device=dev)
+    _check_tensor(out, "out", 1)
+    L = lib()
+    nbytes = L.lift_atax_workspace_bytes(m, n)
+    with torch.cuda.device(dev):
+        ws = _workspace("atax", dev, nbytes, zero=False)
+        check(L.lift_atax_algo_run(_ALGOS[algo], m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(),
+                                   ws.numel(), _stream(dev)))
+    return out

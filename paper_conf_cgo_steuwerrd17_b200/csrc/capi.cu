@@ -1,0 +1,222 @@
+// capi.cu — the C ABI of include/lift.h: host-side validation, device
+// configuration and dispatch to the kernels.  Validation never touches CUDA,
+// so every error path is testable without a GPU.
+#include <limits.h>
+#include <stdio.h>
+#include <string.h>
+
+#include <mutex>
+
+#include "../../include/lift.h"
+#include "../../include/lift_tuning.h"
+#include "launch.h"
+
+namespace lift {
+
+static std::mutex g_dev_mu;
+static DeviceInfo g_dev[64];
+
+cudaError_t device_info(DeviceInfo *out) {
+    int dev = 0;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e != cudaSuccess) return e;
+    if (dev < 0 || dev >= 64) return cudaErrorInvalidDevice;
+    std::lock_guard<std::mutex> lk(g_dev_mu);
+    DeviceInfo &d = g_dev[dev];
+    if (d.device != dev) {
+        DeviceInfo t;
+        t.device = dev;
+        if ((e = cudaDeviceGetAttribute(&t.sms, cudaDevAttrMultiProcessorCount, dev)) != cudaSuccess) return e;
+        if ((e = cudaDeviceGetAttribute(&t.smem_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev)) != cudaSuccess)
+            return e;
+        if ((e = cudaDeviceGetAttribute(&t.smem_per_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev)) !=
+            cudaSuccess)
+            return e;
+        if ((e = cudaDeviceGetAttribute(&t.max_threads_sm, cudaDevAttrMaxThreadsPerMultiProcessor, dev)) !=
+            cudaSuccess)
+            return e;
+        if ((e = cudaDeviceGetAttribute(&t.regs_per_sm, cudaDevAttrMaxRegistersPerMultiprocessor, dev)) !=
+            cudaSuccess)
+            return e;
+        d = t;
+    }
+    *out = d;
+    return cudaSuccess;
+}
+
+}  // namespace lift
+
+using lift::DeviceInfo;
+
+static thread_local char g_cuda_err[256] = "no error";
+
+static int cuda_status(cudaError_t e) {
+    if (e == cudaSuccess) return LIFT_OK;
+    snprintf(g_cuda_err, sizeof g_cuda_err, "%s: %s", cudaGetErrorName(e), cudaGetErrorString(e));
+    return LIFT_ERR_CUDA;
+}
+
+// ---------------------------------------------------------------------------
+// validation helpers (pure host logic)
+// ---------------------------------------------------------------------------
+struct Range {
+    uintptr_t lo, hi;  // [lo, hi)
+};
+static Range rng(const void *p, uint64_t bytes) {
+    uintptr_t a = reinterpret_cast<uintptr_t>(p);
+    return Range{a, a + (uintptr_t)bytes};
+}
+static bool overlap(Range a, Range b) {
+    if (a.lo == a.hi || b.lo == b.hi) return false;
+    return a.lo < b.hi && b.lo < a.hi;
+}
+static bool mis4(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 3) != 0; }
+
+// elements m*n with 4-byte elements must be addressable in int64 bytes
+static bool size_ok(int64_t m, int64_t n) {
+    if (m < 0 || n < 0) return false;
+    if (m == 0 || n == 0) return true;
+    return m <= (INT64_MAX / 4) / n;
+}
+
+extern "C" {
+
+size_t lift_dot_workspace_bytes(int64_t n) {
+    (void)n;
+    return lift::kDotTicketBytes + (size_t)lift::kDotMaxBlocks * sizeof(float);
+}
+
+int lift_dot(int64_t n, const float *x, const float *y, float *result, void *workspace, size_t workspace_bytes,
+             lift_stream_t stream) {
+    if (!size_ok(n, 1)) return LIFT_ERR_BAD_SIZE;
+    if (result == nullptr) return LIFT_ERR_NULL_PTR;
+    if (n > 0 && (x == nullptr || y == nullptr)) return LIFT_ERR_NULL_PTR;
+    if (mis4(result) || (n > 0 && (mis4(x) || mis4(y)))) return LIFT_ERR_MISALIGNED;
+    if (workspace == nullptr || workspace_bytes < lift_dot_workspace_bytes(n) ||
+        (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const Range rr = rng(result, 4), rw = rng(workspace, workspace_bytes);
+    const Range rx = rng(x, (uint64_t)n * 4), ry = rng(y, (uint64_t)n * 4);
+    if (overlap(rr, rx) || overlap(rr, ry) || overlap(rr, rw) || overlap(rw, rx) || overlap(rw, ry))
+        return LIFT_ERR_ALIAS;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    return cuda_status(lift::launch_dot(d, n, x, y, result, workspace, (cudaStream_t)stream));
+}
+
+static int check_gemv_family(int64_t m, int64_t n, const float *A, const float *B, bool two, const float *x,
+                             const float *y) {
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (m > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
+    if (m > 0 && n > 0 && (A == nullptr || x == nullptr || (two && B == nullptr))) return LIFT_ERR_NULL_PTR;
+    if (m > 0 && mis4(y)) return LIFT_ERR_MISALIGNED;
+    if (m > 0 && n > 0 && (mis4(A) || mis4(x) || (two && mis4(B)))) return LIFT_ERR_MISALIGNED;
+    if (m > 0) {
+        const Range ry = rng(y, (uint64_t)m * 4);
+        const uint64_t mat = (uint64_t)m * (uint64_t)n * 4;
+        if (overlap(ry, rng(A, mat)) || overlap(ry, rng(x, (uint64_t)n * 4)) || (two && overlap(ry, rng(B, mat))))
+            return LIFT_ERR_ALIAS;
+    }
+    return LIFT_OK;
+}
+
+int lift_gemv_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y, int wpr, int rg, int blocks,
+                    int xsmem, lift_stream_t stream) {
+    int st = check_gemv_family(m, n, A, nullptr, false, x, y);
+    if (st != LIFT_OK) return st;
+    if (m == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    lift::GemvConfig cfg;
+    cfg.wpr = wpr;
+    cfg.rg = rg;
+    cfg.blocks = blocks;
+    cfg.xsmem = xsmem;
+    return cuda_status(lift::launch_gemv(d, 1, m, n, A, nullptr, x, y, 1.f, 0.f, cfg, (cudaStream_t)stream));
+}
+
+int lift_gemv(int64_t m, int64_t n, const float *A, const float *x, float *y, lift_stream_t stream) {
+    return lift_gemv_tuned(m, n, A, x, y, 0, 0, 0, -1, stream);
+}
+
+int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B, const float *x,
+                       float *y, int wpr, int rg, int blocks, int xsmem, lift_stream_t stream) {
+    int st = check_gemv_family(m, n, A, B, true, x, y);
+    if (st != LIFT_OK) return st;
+    if (m == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    lift::GemvConfig cfg;
+    cfg.wpr = wpr;
+    cfg.rg = rg;
+    cfg.blocks = blocks;
+    cfg.xsmem = xsmem;
+    return cuda_status(lift::launch_gemv(d, 2, m, n, A, B, x, y, alpha, beta, cfg, (cudaStream_t)stream));
+}
+
+int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B, const float *x,
+                 float *y, lift_stream_t stream) {
+    return lift_gesummv_tuned(m, n, alpha, A, beta, B, x, y, 0, 0, 0, -1, stream);
+}
+
+size_t lift_atax_workspace_bytes(int64_t m, int64_t n) {
+    if (!size_ok(m, n)) return 0;
+    size_t a = lift::atax_twopass_ws_bytes(m, n), b = lift::atax_fused_ws_bytes(m, n);
+    return a > b ? a : b;
+}
+
+int lift_atax_algo_run(int algo, int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
+                       size_t workspace_bytes, lift_stream_t stream) {
+    if (algo < LIFT_ATAX_AUTO || algo > LIFT_ATAX_TWOPASS) return LIFT_ERR_BAD_SIZE;
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (n > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
+    if (m > 0 && n > 0 && (A == nullptr || x == nullptr)) return LIFT_ERR_NULL_PTR;
+    if (n > 0 && mis4(y)) return LIFT_ERR_MISALIGNED;
+    if (m > 0 && n > 0 && (mis4(A) || mis4(x))) return LIFT_ERR_MISALIGNED;
+    if (workspace == nullptr || workspace_bytes < lift_atax_workspace_bytes(m, n) ||
+        (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const uint64_t mat = (uint64_t)m * (uint64_t)n * 4;
+    const Range ry = rng(y, (uint64_t)n * 4), rw = rng(workspace, workspace_bytes);
+    const Range rA = rng(A, mat), rx = rng(x, (uint64_t)n * 4);
+    if (overlap(ry, rA) || overlap(ry, rx) || overlap(ry, rw) || overlap(rw, rA) || overlap(rw, rx))
+        return LIFT_ERR_ALIAS;
+    const bool aligned = ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
+                           reinterpret_cast<uintptr_t>(y)) & 15) == 0;
+    const bool fused_ok = lift::atax_fused_supported(m, n, aligned);
+    if (algo == LIFT_ATAX_FUSED && !fused_ok && m > 0 && n > 0) return LIFT_ERR_BAD_SIZE;
+    if (n == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    const bool fused = (algo == LIFT_ATAX_FUSED) || (algo == LIFT_ATAX_AUTO && fused_ok);
+    if (fused) return cuda_status(lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream));
+    return cuda_status(lift::launch_atax_twopass(d, m, n, A, x, y, workspace, (cudaStream_t)stream));
+}
+
+int lift_atax(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
+              size_t workspace_bytes, lift_stream_t stream) {
+    return lift_atax_algo_run(LIFT_ATAX_AUTO, m, n, A, x, y, workspace, workspace_bytes, stream);
+}
+
+const char *lift_strerror(int status) {
+    switch (status) {
+        case LIFT_OK: return "LIFT_OK: success";
+        case LIFT_ERR_NULL_PTR: return "LIFT_ERR_NULL_PTR: a required pointer is NULL";
+        case LIFT_ERR_BAD_SIZE: return "LIFT_ERR_BAD_SIZE: negative or overflowing size, or unsupported shape";
+        case LIFT_ERR_MISALIGNED: return "LIFT_ERR_MISALIGNED: pointer not 4-byte aligned";
+        case LIFT_ERR_ALIAS: return "LIFT_ERR_ALIAS: output overlaps an input or the workspace";
+        case LIFT_ERR_WORKSPACE: return "LIFT_ERR_WORKSPACE: workspace NULL, too small or not 16-byte aligned";
+        case LIFT_ERR_CUDA: return "LIFT_ERR_CUDA: CUDA launch error (see lift_last_cuda_error)";
+        default: return "unknown lift status";
+    }
+}
+
+const char *lift_last_cuda_error(void) { return g_cuda_err; }
+
+int lift_version(void) { return (1 << 16) | 0; }
+
+}  // extern "C"

@@ -1,0 +1,160 @@
+// common.cuh — sm_100a device helpers shared by the Lift hot-path kernels.
+//
+// Vocabulary follows the paper (Sec. 3.2):
+//   reduceSeq  (L320)      per-thread sequential fold in registers
+//   iterate    (L312-324)  the in-block tree (here: warp butterfly + smem)
+//   toLocal    (L368-377)  shared memory; toPrivate = registers
+//   asVector4  (L378-389)  128-bit float4 accesses
+#pragma once
+
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+namespace lift {
+
+constexpr int kWarp = 32;
+
+// ---------------------------------------------------------------------------
+// Global loads
+// ---------------------------------------------------------------------------
+
+// Streaming 128-bit read-only load: the big operand (A, B, x/y of dot) is
+// touched exactly once, so do not allocate it in L1.
+__device__ __forceinline__ float4 ld_stream4(const float4 *p) {
+    float4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.f32 {%0,%1,%2,%3}, [%4];"
+                 : "=f"(r.x), "=f"(r.y), "=f"(r.z), "=f"(r.w)
+                 : "l"(p));
+    return r;
+}
+
+__device__ __forceinline__ float ld_stream1(const float *p) {
+    float r;
+    asm volatile("ld.global.nc.L1::no_allocate.f32 %0, [%1];" : "=f"(r) : "l"(p));
+    return r;
+}
+
+// Read-only cached loads for small operands reused by many threads (x, t).
+__device__ __forceinline__ float4 ld_ro4(const float4 *p) { return __ldg(p); }
+__device__ __forceinline__ float ld_ro1(const float *p) { return __ldg(p); }
+
+// ---------------------------------------------------------------------------
+// multAndSumUp (L767, Fig. 7 l.12 = L959): acc + a*b with one rounding (FMA)
+// — reading R2 — applied per float4 component (mapVec, L381-383).
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ void fma4(float4 &acc, const float4 a, const float4 b) {
+    acc.x = __fmaf_rn(a.x, b.x, acc.x);
+    acc.y = __fmaf_rn(a.y, b.y, acc.y);
+    acc.z = __fmaf_rn(a.z, b.z, acc.z);
+    acc.w = __fmaf_rn(a.w, b.w, acc.w);
+}
+
+__device__ __forceinline__ void fma4s(float4 &acc, const float4 a, const float s) {
+    acc.x = __fmaf_rn(a.x, s, acc.x);
+    acc.y = __fmaf_rn(a.y, s, acc.y);
+    acc.z = __fmaf_rn(a.z, s, acc.z);
+    acc.w = __fmaf_rn(a.w, s, acc.w);
+}
+
+// Fixed-shape fold of the four component accumulators: (x + y) + (z + w).
+__device__ __forceinline__ float hsum4(const float4 v) {
+    return __fadd_rn(__fadd_rn(v.x, v.y), __fadd_rn(v.z, v.w));
+}
+
+__device__ __forceinline__ float4 zero4() { return make_float4(0.f, 0.f, 0.f, 0.f); }
+
+// ---------------------------------------------------------------------------
+// In-warp tree (the iterate-over-local-memory step of Listing 1,
+// done with register shuffles instead of local memory + barriers, Sec. 5.4).
+// Butterfly: every lane ends with the same bits (fp add is commutative).
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ float warp_sum(float v) {
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) v = __fadd_rn(v, __shfl_xor_sync(0xffffffffu, v, o));
+    return v;
+}
+
+// Pairwise (adjacent) tree over a power-of-two number of values in order:
+// out = ((v0+v1)+(v2+v3)) + ...  — Listing 1's iterate over split2.
+template <int N>
+__device__ __forceinline__ float pair_tree(const float *v) {
+    if constexpr (N == 1) {
+        return v[0];
+    } else {
+        float t[N / 2];
+#pragma unroll
+        for (int i = 0; i < N / 2; ++i) t[i] = __fadd_rn(v[2 * i], v[2 * i + 1]);
+        return pair_tree<N / 2>(t);
+    }
+}
+
+// ---------------------------------------------------------------------------
+// mbarrier + 1-D bulk copy (TMA engine; SASS UBLKCP) for staging x in smem.
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ uint32_t smem_u32(const void *p) {
+    return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+
+__device__ __forceinline__ void mbar_init(uint64_t *bar, uint32_t count) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
+}
+
+__device__ __forceinline__ void fence_mbar_init() {
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+}
+
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t *bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+                 : "memory");
+}
+
+__device__ __forceinline__ void mbar_wait_parity(uint64_t *bar, uint32_t parity) {
+    asm volatile(
+        "{\n"
+        ".reg .pred p;\n"
+        "LIFT_WAIT_%=:\n"
+        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+        "@!p bra LIFT_WAIT_%=;\n"
+        "}\n" ::"r"(smem_u32(bar)),
+        "r"(parity)
+        : "memory");
+}
+
+// global -> shared bulk copy; bytes % 16 == 0, both addresses 16-B aligned.
+__device__ __forceinline__ void bulk_g2s(void *dst_smem, const void *src_gmem, uint32_t bytes, uint64_t *bar) {
+    asm volatile(
+        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+            smem_u32(dst_smem)),
+        "l"(src_gmem), "r"(bytes), "r"(smem_u32(bar))
+        : "memory");
+}
+
+// Stage `bytes` (multiple of 16) of gmem into smem with the bulk-copy engine.
+// Called by ALL threads of the block; thread 0 issues. Returns after the data
+// has landed (mbarrier phase 0 completes).  `bar` must be a fresh mbarrier
+// slot in shared memory.  Work independent of the staged data may be issued
+// by the caller before calling stage_wait().
+__device__ __forceinline__ void stage_issue(void *dst, const void *src, uint32_t bytes, uint64_t *bar) {
+    if (threadIdx.x == 0) {
+        mbar_init(bar, 1);
+        fence_mbar_init();
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        mbar_arrive_expect_tx(bar, bytes);
+        constexpr uint32_t kChunk = 32768;
+        for (uint32_t off = 0; off < bytes; off += kChunk) {
+            uint32_t b = bytes - off < kChunk ? bytes - off : kChunk;
+            bulk_g2s(static_cast<char *>(dst) + off, static_cast<const char *>(src) + off, b, bar);
+        }
+    }
+}
+
+__device__ __forceinline__ void stage_wait(uint64_t *bar) { mbar_wait_parity(bar, 0); }
+
+// Named barrier over `nthreads` threads (multiple of 32) with id in [1, 15].
+__device__ __forceinline__ void named_bar_sync(int id, int nthreads) {
+    asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
+}
+
+}  // namespace lift

@@ -1,0 +1,136 @@
+// dot.cu — k_dot: dot(x, y) = reduce(+, 0, map(x, zip(x, y)))
+//
+// One launch does all three stages of Listing 1 (L391-401) plus the second
+// kernel the paper omits (L422-426):
+//   (1) zip + map + reduceSeq(multAndSumUp, 0): each thread folds a strided
+//       chunk of float4 pairs into U independent float4 accumulators
+//       (asVector4, L378-389; Fig. 7 l.10-14 = L957-961).  No product array
+//       is ever formed (views instead of intermediates, L164-170).
+//   (2) in-block tree (iterate, L394-397): warp butterfly, then one smem
+//       exchange across warps (one barrier, Sec. 5.4).
+//   (3) multi-stage: every block writes its partial (toGlobal, L393); the
+//       LAST block to arrive (atomic ticket) sums all partials in a fixed
+//       order and writes the scalar, then re-arms the ticket.
+// mapWrg over chunks (Fig. 7 l.7-8 = L954-955) becomes a persistent
+// grid-stride loop over a grid sized from the SM count.
+#include "common.cuh"
+#include "launch.h"
+
+namespace lift {
+
+template <int TPB, int U>
+__device__ __forceinline__ float block_sum(float v, float *red) {
+    constexpr int W = TPB / kWarp;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    v = warp_sum(v);
+    if (lane == 0) red[warp] = v;
+    __syncthreads();
+    float r = 0.f;
+    if (warp == 0) {
+        r = lane < W ? red[lane] : 0.f;
+        r = warp_sum(r);
+    }
+    return r;  // valid in warp 0
+}
+
+template <int TPB, int U, bool VEC>
+__global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict__ x, const float *__restrict__ y,
+                                             float *__restrict__ result, float *__restrict__ partials,
+                                             unsigned int *__restrict__ ticket) {
+    __shared__ float red[TPB / kWarp];
+    __shared__ bool am_last;
+    const int64_t stride = (int64_t)gridDim.x * TPB;
+    int64_t i = (int64_t)blockIdx.x * TPB + threadIdx.x;
+    float s;
+    if constexpr (VEC) {
+        const int64_t n4 = n >> 2;
+        const float4 *x4 = reinterpret_cast<const float4 *>(x);
+        const float4 *y4 = reinterpret_cast<const float4 *>(y);
+        float4 acc[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) acc[u] = zero4();
+        // reduceSeq over this thread's chunk, U float4 pairs in flight per stream
+        for (; i + (U - 1) * stride < n4; i += U * stride) {
+            float4 a[U], b[U];
+#pragma unroll
+            for (int u = 0; u < U; ++u) {
+                a[u] = ld_stream4(x4 + i + u * stride);
+                b[u] = ld_stream4(y4 + i + u * stride);
+            }
+#pragma unroll
+            for (int u = 0; u < U; ++u) fma4(acc[u], a[u], b[u]);
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            if (i + u * stride < n4) fma4(acc[u], ld_stream4(x4 + i + u * stride), ld_stream4(y4 + i + u * stride));
+        }
+        float h[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) h[u] = hsum4(acc[u]);
+        s = pair_tree<U>(h);
+        // scalar tail (n % 4 elements) folded by block 0
+        if (blockIdx.x == 0 && threadIdx.x < (n & 3)) {
+            const int64_t e = (n4 << 2) + threadIdx.x;
+            s = __fmaf_rn(ld_ro1(x + e), ld_ro1(y + e), s);
+        }
+    } else {
+        float acc[4] = {0.f, 0.f, 0.f, 0.f};
+        for (; i + 3 * stride < n; i += 4 * stride) {
+            float a[4], b[4];
+#pragma unroll
+            for (int u = 0; u < 4; ++u) {
+                a[u] = ld_stream1(x + i + u * stride);
+                b[u] = ld_stream1(y + i + u * stride);
+            }
+#pragma unroll
+            for (int u = 0; u < 4; ++u) acc[u] = __fmaf_rn(a[u], b[u], acc[u]);
+        }
+#pragma unroll
+        for (int u = 0; u < 4; ++u)
+            if (i + u * stride < n) acc[u] = __fmaf_rn(ld_stream1(x + i + u * stride), ld_stream1(y + i + u * stride), acc[u]);
+        s = pair_tree<4>(acc);
+    }
+
+    float bs = block_sum<TPB, U>(s, red);
+    if (threadIdx.x == 0) {
+        partials[blockIdx.x] = bs;
+        __threadfence();
+        const unsigned int t = atomicAdd(ticket, 1u);
+        am_last = (t == gridDim.x - 1);
+    }
+    __syncthreads();
+    if (!am_last) return;
+    // second stage (L422-426), fixed order: thread j folds partials j, j+TPB, ...
+    __threadfence();
+    float p = 0.f;
+    for (int j = threadIdx.x; j < (int)gridDim.x; j += TPB) p = __fadd_rn(p, __ldcg(partials + j));
+    __syncthreads();  // red[] reuse
+    float tot = block_sum<TPB, U>(p, red);
+    if (threadIdx.x == 0) {
+        *result = tot;
+        *ticket = 0u;  // re-arm for the next launch on this workspace
+    }
+}
+
+cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
+                       void *workspace, cudaStream_t s) {
+    constexpr int TPB = 512;
+    constexpr int U = 4;
+    unsigned int *ticket = static_cast<unsigned int *>(workspace);
+    float *partials = reinterpret_cast<float *>(static_cast<char *>(workspace) + kDotTicketBytes);
+    const bool vec = ((reinterpret_cast<uintptr_t>(x) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
+    const int64_t units = vec ? (n >> 2) : n;
+    // enough blocks to give every thread >= 1 unit; at most a full resident wave
+    const int per_sm = 2048 / TPB;
+    int64_t want = (units + TPB - 1) / TPB;
+    int64_t cap = (int64_t)d.sms * per_sm;
+    if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;
+    int blocks = (int)(want < 1 ? 1 : (want > cap ? cap : want));
+    if (vec)
+        k_dot<TPB, U, true><<<blocks, TPB, 0, s>>>(n, x, y, result, partials, ticket);
+    else
+        k_dot<TPB, U, false><<<blocks, TPB, 0, s>>>(n, x, y, result, partials, ticket);
+    return cudaGetLastError();
+}
+
+}  // namespace lift

@@ -1,0 +1,280 @@
+// gemv.cu — k_gemv: GEMV y = A x and GESUMMV y = alpha A x + beta B x
+// (Table 1), the zip -> map(x) -> reduce(+) kernel
+// applied per row with x reused across rows.
+//
+// Mapping of the Lift patterns onto sm_100a:
+//   mapWrg over rows (L359-367)     persistent grid-stride loop over row groups
+//   toLocal(x) (L368-377)           x staged ONCE per block into smem by the
+//                                   bulk-copy engine (cp.async.bulk + mbarrier,
+//                                   SASS UBLKCP), overlapped with the first A loads
+//   zip(A_i, x) / asVector4          128-bit streaming loads of A (no L1 alloc)
+//   reduceSeq(multAndSumUp) (L320)   per-lane FMA fold in registers
+//   iterate tree (L394-397)          warp butterfly + fixed pairwise tree
+//   GESUMMV's zip of (A_i, B_i)      two accumulator sets, one pass, y_i =
+//                                    alpha*sA + beta*sB: Ax and Bx never exist
+//
+// Canonical per-row order (independent of m, of the launch configuration and
+// of row sharding): a row of nv = n/VEC vectors is cut into 8 "slices" of
+// 32 virtual lanes.  Virtual lane v = 32*p + l (slice p, lane l) folds the
+// vectors j = v, v + 256, v + 512, ... in increasing j into one accumulator
+// (per component for float4), starting from 0.  Each virtual lane's value is
+// (acc.x + acc.y) + (acc.z + acc.w); each slice is a 32-lane butterfly; the
+// row is the pairwise tree over the 8 slices.  A block row group of WPR warps
+// computes 8/WPR slices per warp, so every WPR gives the same bits.
+#include "common.cuh"
+#include "launch.h"
+
+namespace lift {
+
+constexpr int kSlices = 8;
+constexpr int kVLanes = kSlices * kWarp;  // 256 virtual lanes per row
+
+template <int VEC>
+struct Vec;
+template <>
+struct Vec<4> {
+    using T = float4;
+    static __device__ __forceinline__ T zero() { return zero4(); }
+    static __device__ __forceinline__ T ld_stream(const float *base, int64_t j) {
+        return ld_stream4(reinterpret_cast<const float4 *>(base) + j);
+    }
+    static __device__ __forceinline__ T ld_x(const float *base, int64_t j) {
+        return reinterpret_cast<const float4 *>(base)[j];
+    }
+    static __device__ __forceinline__ T ld_x_global(const float *base, int64_t j) {
+        return ld_ro4(reinterpret_cast<const float4 *>(base) + j);
+    }
+    static __device__ __forceinline__ void fma(T &acc, T a, T b) { fma4(acc, a, b); }
+    static __device__ __forceinline__ float hsum(T v) { return hsum4(v); }
+};
+template <>
+struct Vec<1> {
+    using T = float;
+    static __device__ __forceinline__ T zero() { return 0.f; }
+    static __device__ __forceinline__ T ld_stream(const float *base, int64_t j) { return ld_stream1(base + j); }
+    static __device__ __forceinline__ T ld_x(const float *base, int64_t j) { return base[j]; }
+    static __device__ __forceinline__ T ld_x_global(const float *base, int64_t j) { return ld_ro1(base + j); }
+    static __device__ __forceinline__ void fma(T &acc, T a, T b) { acc = __fmaf_rn(a, b, acc); }
+    static __device__ __forceinline__ float hsum(T v) { return v; }
+};
+
+// smem layout: [mbarrier 16 B][red: 2 buffers x RG x NMAT x 8 floats][x: n floats, 16-B aligned]
+template <int NMAT, int RG>
+__host__ __device__ constexpr int gemv_red_bytes() {
+    return 2 * RG * NMAT * kSlices * 4;
+}
+template <int NMAT, int RG>
+__host__ __device__ constexpr int gemv_x_offset() {
+    return (16 + gemv_red_bytes<NMAT, RG>() + 15) / 16 * 16;
+}
+
+template <int NMAT, int VEC, int WPR, int RG, bool XSMEM>
+__global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, const float *__restrict__ A,
+                                                        const float *__restrict__ B, const float *__restrict__ x,
+                                                        float *__restrict__ y, float alpha, float beta) {
+    using V = Vec<VEC>;
+    using T = typename V::T;
+    constexpr int KQ = kSlices / WPR;                                    // slices per warp
+    constexpr int UK = (8 / (KQ * NMAT)) > 0 ? (8 / (KQ * NMAT)) : 1;  // k-steps per batch
+    extern __shared__ __align__(16) unsigned char smem[];
+    uint64_t *bar = reinterpret_cast<uint64_t *>(smem);
+    float *red = reinterpret_cast<float *>(smem + 16);
+    float *xs = reinterpret_cast<float *>(smem + gemv_x_offset<NMAT, RG>());
+
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int g = warp / WPR;   // row group inside the block
+    const int wr = warp % WPR;  // warp rank inside the row group
+    const int64_t nv = n / VEC;
+    const int64_t kcount = (nv + kVLanes - 1) / kVLanes;
+
+    bool x_pending = false;
+    if constexpr (XSMEM) {
+        stage_issue(xs, x, (uint32_t)(n * 4), bar);  // toLocal(x), one bulk copy per block
+        x_pending = true;
+    }
+
+    const int64_t row_step = (int64_t)gridDim.x * RG;
+    int buf = 0;
+    for (int64_t row = (int64_t)blockIdx.x * RG + g; row < m; row += row_step, buf ^= 1) {
+        T acc[NMAT][KQ];
+#pragma unroll
+        for (int mt = 0; mt < NMAT; ++mt)
+#pragma unroll
+            for (int q = 0; q < KQ; ++q) acc[mt][q] = V::zero();
+        const float *Ar = A + row * n;
+        const float *Br = (NMAT == 2) ? B + row * n : nullptr;
+
+        for (int64_t k0 = 0; k0 < kcount; k0 += UK) {
+            T a[NMAT][UK][KQ];
+            bool ok[UK][KQ];
+#pragma unroll
+            for (int u = 0; u < UK; ++u)
+#pragma unroll
+                for (int q = 0; q < KQ; ++q) {
+                    const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
+                    ok[u][q] = (k0 + u < kcount) && (j < nv);
+#pragma unroll
+                    for (int mt = 0; mt < NMAT; ++mt)
+                        a[mt][u][q] = ok[u][q] ? V::ld_stream(mt == 0 ? Ar : Br, j) : V::zero();
+                }
+            if constexpr (XSMEM) {
+                if (x_pending) {  // first batch: A loads are in flight, now wait for x
+                    stage_wait(bar);
+                    x_pending = false;
+                }
+            }
+#pragma unroll
+            for (int u = 0; u < UK; ++u)
+#pragma unroll
+                for (int q = 0; q < KQ; ++q) {
+                    const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
+                    T xv = V::zero();
+                    if (ok[u][q]) {
+                        if constexpr (XSMEM)
+                            xv = V::ld_x(xs, j);
+                        else
+                            xv = V::ld_x_global(x, j);
+                    }
+#pragma unroll
+                    for (int mt = 0; mt < NMAT; ++mt) V::fma(acc[mt][q], a[mt][u][q], xv);
+                }
+        }
+
+        // slice values (butterfly), then the pairwise tree over the 8 slices
+        float w[NMAT][KQ];
+#pragma unroll
+        for (int mt = 0; mt < NMAT; ++mt)
+#pragma unroll
+            for (int q = 0; q < KQ; ++q) w[mt][q] = warp_sum(V::hsum(acc[mt][q]));
+
+        float s[NMAT];
+        bool writer;
+        if constexpr (WPR == 1) {
+#pragma unroll
+            for (int mt = 0; mt < NMAT; ++mt) s[mt] = pair_tree<kSlices>(w[mt]);
+            writer = (lane == 0);
+        } else {
+            float *r = red + ((buf * RG + g) * NMAT) * kSlices;
+            if (lane == 0) {
+#pragma unroll
+                for (int mt = 0; mt < NMAT; ++mt)
+#pragma unroll
+                    for (int q = 0; q < KQ; ++q) r[mt * kSlices + wr * KQ + q] = w[mt][q];
+            }
+            if constexpr (RG == 1)
+                __syncthreads();
+            else
+                named_bar_sync(1 + g, WPR * kWarp);
+            writer = (wr == 0 && lane == 0);
+            if (writer) {
+#pragma unroll
+                for (int mt = 0; mt < NMAT; ++mt) {
+                    float v[kSlices];
+#pragma unroll
+                    for (int p = 0; p < kSlices; ++p) v[p] = r[mt * kSlices + p];
+                    s[mt] = pair_tree<kSlices>(v);
+                }
+            }
+        }
+        if (writer) {
+            if constexpr (NMAT == 1)
+                y[row] = s[0];
+            else
+                y[row] = __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, s[1]));
+        }
+    }
+    if constexpr (XSMEM) {
+        // a block that received no row must still retire its bulk copy
+        if (x_pending) stage_wait(bar);
+    }
+}
+
+// ---------------------------------------------------------------------------
+// host-side configuration
+// ---------------------------------------------------------------------------
+
+template <int NMAT, int VEC, int WPR, int RG, bool XSMEM>
+static cudaError_t run_gemv(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *B,
+                            const float *x, float *y, float alpha, float beta, int blocks, cudaStream_t s) {
+    auto kern = k_gemv<NMAT, VEC, WPR, RG, XSMEM>;
+    constexpr int threads = RG * WPR * kWarp;
+    size_t smem = gemv_x_offset<NMAT, RG>() + (XSMEM ? (size_t)n * 4 : 0);
+    if (smem > 48 * 1024) {
+        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        if (e != cudaSuccess) return e;
+    }
+    int per_sm = 0;
+    cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, threads, smem);
+    if (e != cudaSuccess) return e;
+    if (per_sm < 1) return cudaErrorInvalidConfiguration;
+    const int64_t groups = (m + RG - 1) / RG;
+    int64_t cap = (int64_t)per_sm * d.sms;
+    int64_t g = blocks > 0 ? blocks : (groups < cap ? groups : cap);
+    if (g < 1) g = 1;
+    kern<<<(unsigned)g, threads, smem, s>>>(m, n, A, B, x, y, alpha, beta);
+    return cudaGetLastError();
+}
+
+template <int NMAT, int VEC, bool XSMEM>
+static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int64_t m, int64_t n, const float *A,
+                                const float *B, const float *x, float *y, float alpha, float beta, int blocks,
+                                cudaStream_t s) {
+    // block = RG row groups of WPR warps; 256..1024 threads
+#define LIFT_GEMV_CASE(W, R)                                                                     \
+    if (wpr == W && rg == R)                                                                     \
+        return run_gemv<NMAT, VEC, W, R, XSMEM>(d, m, n, A, B, x, y, alpha, beta, blocks, s);
+    LIFT_GEMV_CASE(8, 1)
+    LIFT_GEMV_CASE(8, 2)
+    LIFT_GEMV_CASE(8, 4)
+    LIFT_GEMV_CASE(4, 2)
+    LIFT_GEMV_CASE(4, 4)
+    LIFT_GEMV_CASE(4, 8)
+    LIFT_GEMV_CASE(2, 4)
+    LIFT_GEMV_CASE(2, 8)
+    LIFT_GEMV_CASE(1, 8)
+    LIFT_GEMV_CASE(1, 16)
+    LIFT_GEMV_CASE(1, 32)
+#undef LIFT_GEMV_CASE
+    return cudaErrorInvalidValue;
+}
+
+cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, const float *A, const float *B,
+                        const float *x, float *y, float alpha, float beta, GemvConfig cfg, cudaStream_t s) {
+    if (m == 0) return cudaSuccess;
+    if (n == 0) return cudaMemsetAsync(y, 0, (size_t)m * sizeof(float), s);
+    uintptr_t orr = reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
+                    (nmat == 2 ? reinterpret_cast<uintptr_t>(B) : 0);
+    const bool vec = (n % 4 == 0) && (orr & 15) == 0;
+    // x in smem when it fits next to the red buffers (bulk copy needs 16-B units)
+    const size_t x_bytes = (size_t)n * 4;
+    bool xsmem = vec && x_bytes + 1024 <= (size_t)d.smem_optin;
+    if (cfg.xsmem == 0) xsmem = false;
+    if (cfg.xsmem == 1 && !xsmem) return cudaErrorInvalidValue;
+
+    int wpr = cfg.wpr, rg = cfg.rg;
+    if (wpr == 0) {
+        // spread rows over enough warps to fill the chip: about 32 resident
+        // warps per SM want a row task each
+        const int64_t want_tasks = (int64_t)d.sms * 32;
+        wpr = 1;
+        while (wpr < 8 && m * wpr < want_tasks) wpr *= 2;
+        if (!vec) wpr = 1;
+    }
+    if (rg == 0) {
+        // 256-thread blocks by default; 1024 when one block per SM holds a large x
+        rg = 256 / (wpr * kWarp);
+        if (xsmem && 2 * (x_bytes + 1024) > (size_t)d.smem_per_sm) rg = 1024 / (wpr * kWarp);
+        if (rg < 1) rg = 1;
+    }
+    if (vec) {
+        if (nmat == 1)
+            return xsmem ? dispatch_wpr<1, 4, true>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
+                         : dispatch_wpr<1, 4, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+        return xsmem ? dispatch_wpr<2, 4, true>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
+                     : dispatch_wpr<2, 4, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+    }
+    if (nmat == 1) return dispatch_wpr<1, 1, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+    return dispatch_wpr<2, 1, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+}
+
+}  // namespace lift

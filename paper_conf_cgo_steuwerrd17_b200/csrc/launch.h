@@ -1,0 +1,49 @@
+// launch.h — internal launcher interface between capi.cu (validation,
+// configuration) and the kernel translation units.  Not part of the C ABI.
+#pragma once
+
+#include <cuda_runtime.h>
+#include <stddef.h>
+#include <stdint.h>
+
+namespace lift {
+
+struct DeviceInfo {
+    int device = -1;
+    int sms = 0;              // cudaDevAttrMultiProcessorCount (148 on B200)
+    int smem_optin = 0;       // max dynamic smem per block (opt-in)
+    int smem_per_sm = 0;      // max smem per SM
+    int max_threads_sm = 0;   // 2048
+    int regs_per_sm = 0;      // 65536
+};
+
+// Cached per device; thread-safe after the first call per device.
+cudaError_t device_info(DeviceInfo *out);
+
+// ---- dot -------------------------------------------------------------------
+constexpr int kDotMaxBlocks = 4096;
+constexpr size_t kDotTicketBytes = 16;
+cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
+                       void *workspace, cudaStream_t s);
+
+// ---- GEMV / GESUMMV ----------------------------------------------------------
+struct GemvConfig {
+    int wpr = 0;     // warps per row   (1, 2, 4, 8); 0 = auto
+    int rg = 0;      // row groups per block; 0 = auto
+    int blocks = 0;  // grid size; 0 = auto (persistent)
+    int xsmem = -1;  // 1 = stage x in smem by bulk copy, 0 = read x through L1, -1 = auto
+};
+// nmat = 1: y = A x;  nmat = 2: y = alpha A x + beta B x
+cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, const float *A, const float *B,
+                        const float *x, float *y, float alpha, float beta, GemvConfig cfg, cudaStream_t s);
+
+// ---- ATAX ----------------------------------------------------------------------
+size_t atax_twopass_ws_bytes(int64_t m, int64_t n);
+size_t atax_fused_ws_bytes(int64_t m, int64_t n);
+bool atax_fused_supported(int64_t m, int64_t n, bool aligned16);
+cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
+                                float *y, void *ws, cudaStream_t s);
+cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
+                              float *y, void *ws, cudaStream_t s);
+
+}  // namespace lift

@@ -1,0 +1,161 @@
+"""C-ABI library: loads, exports every symbol include/*.h declares, and its
+host-side validation returns the documented status codes before touching
+CUDA.  Pointers here are fake integers: no error path dereferences them."""
+import ctypes
+import subprocess
+
+import pytest
+
+import paper_conf_cgo_steuwerrd17_b200 as lift
+from paper_conf_cgo_steuwerrd17_b200 import _lib
+
+L = lift.lib()
+OK, NULL, SIZE, MIS, ALIAS, WS, CUDA = range(7)
+
+P = 1 << 20  # fake, 256-B aligned "device" addresses far apart
+A_, B_, X_, Y_, W_ = P * 16, P * 64, P * 128, P * 160, P * 192
+
+
+def test_library_exports_every_header_symbol():
+    names = _lib.header_functions()
+    assert {"lift_dot", "lift_gemv", "lift_gesummv", "lift_atax"} <= set(names)
+    out = subprocess.run(["nm", "-D", "--defined-only", lift.library_path()], capture_output=True, text=True,
+                         check=True).stdout
+    exported = {line.split()[-1] for line in out.splitlines() if " T " in line}
+    missing = [n for n in names if n not in exported]
+    assert not missing, missing
+    for n in names:
+        assert hasattr(L, n)
+    assert set(names) == set(_lib.SIGNATURES)
+
+
+def test_exports_nothing_else():
+    out = subprocess.run(["nm", "-D", "--defined-only", lift.library_path()], capture_output=True, text=True,
+                         check=True).stdout
+    exported = {line.split()[-1] for line in out.splitlines() if " T " in line}
+    assert {e for e in exported if e.startswith("lift_")} == set(_lib.header_functions())
+
+
+def test_sm100a_cubin_only():
+    out = subprocess.run(["cuobjdump", "--list-elf", lift.library_path()], capture_output=True, text=True).stdout
+    assert "sm_100a" in out
+    for bad in ("sm_90", "sm_80", "sm_103"):
+        assert bad not in out
+
+
+def test_version_and_strerror():
+    assert L.lift_version() >> 16 == 1
+    for s in range(7):
+        msg = L.lift_strerror(s).decode()
+        assert msg.startswith("LIFT_")
+    assert L.lift_strerror(99).decode() == "unknown lift status"
+
+
+def test_workspace_sizes():
+    assert L.lift_dot_workspace_bytes(0) >= 16 + 4 * 148
+    assert L.lift_dot_workspace_bytes(1 << 31) == L.lift_dot_workspace_bytes(1)
+    w = L.lift_atax_workspace_bytes(8192, 8192)
+    assert w >= 8192 * 4 + 148 * 8192 * 4
+    assert L.lift_atax_workspace_bytes(-1, 5) == 0
+
+
+# ---------------------------------------------------------------- dot
+def test_dot_validation():
+    ws_ok = L.lift_dot_workspace_bytes(100)
+    assert L.lift_dot(-1, X_, Y_, W_ + ws_ok + 64, W_, ws_ok, None) == SIZE
+    assert L.lift_dot(100, None, Y_, P * 300, W_, ws_ok, None) == NULL
+    assert L.lift_dot(100, X_, Y_, None, W_, ws_ok, None) == NULL
+    assert L.lift_dot(100, X_ + 2, Y_, P * 300, W_, ws_ok, None) == MIS
+    assert L.lift_dot(100, X_, Y_, P * 300, None, ws_ok, None) == WS
+    assert L.lift_dot(100, X_, Y_, P * 300, W_, ws_ok - 4, None) == WS
+    assert L.lift_dot(100, X_, Y_, P * 300, W_ + 4, ws_ok, None) == WS
+    assert L.lift_dot(100, X_, Y_, X_ + 8, W_, ws_ok, None) == ALIAS  # result inside x
+    assert L.lift_dot(100, X_, Y_, W_ + 16, W_, ws_ok, None) == ALIAS  # result inside workspace
+    assert L.lift_dot(100, X_, Y_, P * 300, Y_ + 64, ws_ok, None) == ALIAS  # workspace over y
+
+
+# ---------------------------------------------------------------- GEMV family
+def test_gemv_validation():
+    assert L.lift_gemv(-1, 4, A_, X_, Y_, None) == SIZE
+    assert L.lift_gemv(4, -1, A_, X_, Y_, None) == SIZE
+    assert L.lift_gemv(1 << 40, 1 << 40, A_, X_, Y_, None) == SIZE  # m*n*4 overflows
+    assert L.lift_gemv(4, 4, None, X_, Y_, None) == NULL
+    assert L.lift_gemv(4, 4, A_, None, Y_, None) == NULL
+    assert L.lift_gemv(4, 4, A_, X_, None, None) == NULL
+    assert L.lift_gemv(4, 4, A_ + 1, X_, Y_, None) == MIS
+    assert L.lift_gemv(4, 4, A_, X_, Y_ + 2, None) == MIS
+    assert L.lift_gemv(4, 4, A_, X_, A_ + 60, None) == ALIAS
+    assert L.lift_gemv(4, 4, A_, X_, X_ - 4, None) == ALIAS
+    # m == 0 is a no-op that never touches CUDA (even with NULL pointers)
+    assert L.lift_gemv(0, 4, None, None, None, None) == OK
+    # aligned but only 4-byte aligned is accepted (scalar path): must reach CUDA
+    st = L.lift_gemv(4, 3, A_ + 4, X_ + 4, Y_ + 4, None)
+    assert st in (OK, CUDA)
+
+
+def test_gesummv_validation():
+    assert L.lift_gesummv(4, 4, 1.0, A_, 1.0, None, X_, Y_, None) == NULL
+    assert L.lift_gesummv(4, 4, 1.0, A_, 1.0, B_ + 2, X_, Y_, None) == MIS
+    assert L.lift_gesummv(4, 4, 1.0, A_, 1.0, B_, X_, B_ + 4, None) == ALIAS
+    assert L.lift_gesummv(0, 4, 1.0, None, 1.0, None, None, None, None) == OK
+
+
+def test_tuned_validation():
+    assert L.lift_gemv_tuned(-1, 4, A_, X_, Y_, 8, 1, 0, -1, None) == SIZE
+    assert L.lift_gesummv_tuned(4, 4, 1.0, A_, 1.0, B_, X_, A_, 8, 1, 0, -1, None) == ALIAS
+
+
+# ---------------------------------------------------------------- ATAX
+def test_atax_validation():
+    m, n = 64, 32
+    ws = L.lift_atax_workspace_bytes(m, n)
+    assert L.lift_atax(-2, n, A_, X_, Y_, W_, ws, None) == SIZE
+    assert L.lift_atax(m, n, None, X_, Y_, W_, ws, None) == NULL
+    assert L.lift_atax(m, n, A_, X_, None, W_, ws, None) == NULL
+    assert L.lift_atax(m, n, A_, X_ + 1, Y_, W_, ws, None) == MIS
+    assert L.lift_atax(m, n, A_, X_, Y_, None, ws, None) == WS
+    assert L.lift_atax(m, n, A_, X_, Y_, W_, ws - 1, None) == WS
+    assert L.lift_atax(m, n, A_, X_, Y_, W_ + 8, ws, None) == WS
+    assert L.lift_atax(m, n, A_, X_, A_ + 128, W_, ws, None) == ALIAS
+    assert L.lift_atax(m, n, A_, X_, Y_, A_, ws, None) == ALIAS
+    assert L.lift_atax(m, n, A_, X_, Y_, W_ + 8 * 1024 * 1024, ws, None) in (OK, CUDA)  # valid args
+    assert L.lift_atax_algo_run(7, m, n, A_, X_, Y_, W_, ws, None) == SIZE
+    # fused needs n % 4 == 0 and 16-B alignment: refused up front
+    assert L.lift_atax_algo_run(1, m, 33, A_, X_, Y_, W_, L.lift_atax_workspace_bytes(m, 33), None) == SIZE
+    assert L.lift_atax(m, 0, A_, X_, Y_, W_, L.lift_atax_workspace_bytes(m, 0), None) == OK
+
+
+def test_valid_call_without_gpu_fails_loudly():
+    import torch
+
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    st = L.lift_gemv(4, 4, A_, X_, Y_, None)
+    assert st == CUDA
+    assert "cuda" in L.lift_last_cuda_error().decode().lower() or "device" in L.lift_last_cuda_error().decode().lower()
+    with pytest.raises(lift.LiftError):
+        _lib.check(st)
+
+
+def test_python_binding_rejects_cpu_tensors():
+    import torch
+
+    A = torch.zeros(4, 4)
+    x = torch.zeros(4)
+    with pytest.raises(ValueError, match="no CPU path"):
+        lift.lift_gemv(A, x)
+    with pytest.raises(TypeError):
+        lift.lift_gemv(A.double(), x)
+
+
+def test_ctypes_signatures_match_header_arity():
+    import re
+
+    txt = open(_lib._build.INCLUDE + "/lift.h").read() + open(_lib._build.INCLUDE + "/lift_tuning.h").read()
+    txt = re.sub(r"/\*.*?\*/", "", txt, flags=re.S)
+    for name, (_, args) in _lib.SIGNATURES.items():
+        m = re.search(r"\b" + name + r"\s*\(([^)]*)\)", txt)
+        assert m, name
+        params = [p for p in m.group(1).split(",") if p.strip() and p.strip() != "void"]
+        assert len(params) == len(args), (name, params)
+    assert ctypes.sizeof(ctypes.c_size_t) == 8

@@ -1,0 +1,339 @@
+"""GPU parity: the CUDA path (through the C ABI) against the fp64 oracle.
+
+Acceptance (BASELINE.json north_star), elementwise:
+    |y_gpu - y_ref| <= 1e-5 * mag + 1e-6,   mag = sum |terms| (from the oracle)
+Integer-valued / structured inputs whose exact result is reached in fp32 in
+ANY summation order are compared bitwise (SURVEY.md §8(c) pins).
+
+Inputs come from synth (seeded, counter-based): small cases are generated on
+the host and copied; BASELINE-size cases are generated in HBM by torch ops and
+the oracle regenerates the sampled rows on the host from the same counters.
+"""
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import synth
+import paper_conf_cgo_steuwerrd17_b200 as lift
+
+pytestmark = pytest.mark.gpu
+
+ALPHA, BETA = 1.5, 1.2  # bench values (reading R9 / A9)
+
+
+def dev_np(a, device):
+    return torch.from_numpy(np.ascontiguousarray(a)).to(device)
+
+
+def assert_tol(got, ref, mag, what=""):
+    ok, margin = oracle.within_tol(got, ref, mag)
+    assert ok, f"{what}: tolerance margin {margin:.3g} > 1"
+    return margin
+
+
+def rand(seed, shape, dist="sym"):
+    return synth.numpy_uniform(seed, 0, int(np.prod(shape)), dist).reshape(shape)
+
+
+# ===================================================================== dot
+@pytest.mark.parametrize("n", [0, 1, 3, 4, 5, 127, 128, 129, 4097, 1 << 20, (1 << 20) + 3])
+@pytest.mark.parametrize("dist", ["sym", "pos"])
+def test_dot_parity(cuda_device, n, dist):
+    x = rand(synth.SEED_X, (n,), dist)
+    y = rand(synth.SEED_Y, (n,), dist)
+    got = lift.lift_dot(dev_np(x, cuda_device), dev_np(y, cuda_device)).item()
+    ref, mag = oracle.dot(x, y)
+    assert_tol([got], [ref], [mag], f"dot n={n}")
+
+
+@pytest.mark.parametrize("off", [1, 2, 3])
+def test_dot_unaligned_scalar_path(cuda_device, off):
+    n = 10007
+    xb = dev_np(rand(0, (n + off,)), cuda_device)
+    yb = dev_np(rand(1, (n + 4,)), cuda_device)
+    x, y = xb[off:], yb[:n]
+    got = lift.lift_dot(x, y).item()
+    ref, mag = oracle.dot(x.cpu().numpy(), y.cpu().numpy())
+    assert_tol([got], [ref], [mag], "dot unaligned")
+
+
+def test_dot_exact_cases(cuda_device):
+    for n in (1, 1000, 1 << 20, (1 << 24)):
+        ones = torch.ones(n, device=cuda_device)
+        assert lift.lift_dot(ones, ones).item() == float(n)
+    alt = torch.ones(1 << 20, device=cuda_device)
+    alt[1::2] = -1
+    assert lift.lift_dot(alt, torch.ones_like(alt)).item() == 0.0
+    assert lift.lift_dot(torch.zeros(0, device=cuda_device), torch.zeros(0, device=cuda_device)).item() == 0.0
+
+
+def test_dot_deterministic_and_symmetric(cuda_device):
+    n = (1 << 22) + 5
+    x = synth.torch_uniform(0, 0, n, device=cuda_device)
+    y = synth.torch_uniform(1, 0, n, device=cuda_device)
+    a = lift.lift_dot(x, y).item()
+    for _ in range(3):
+        assert lift.lift_dot(x, y).item() == a
+    assert lift.lift_dot(y, x).item() == a
+
+
+def test_dot_ticket_rearms_across_many_calls(cuda_device):
+    # the last-block ticket must return to zero every launch (else results go stale)
+    n = 1 << 16
+    ones = torch.ones(n, device=cuda_device)
+    for k in range(1, 20):
+        v = torch.full((n,), float(k), device=cuda_device)
+        assert lift.lift_dot(v, ones).item() == float(k * n)
+
+
+@pytest.mark.slow
+def test_dot_full_size_2pow31(cuda_device):
+    """configs[4]: 2^31-element dot (one GPU holds 16 GiB of x, y)."""
+    n = 1 << 31
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    y = synth.torch_uniform(synth.SEED_Y, 0, n, device=cuda_device)
+    got = lift.lift_dot(x, y).item()
+    del x, y
+    torch.cuda.empty_cache()
+    ref = 0.0
+    mag = 0.0
+    ch = 1 << 27
+    for s in range(0, n, ch):  # reading A23: chunked fp64 folds agree to ~1e-12
+        r, m = oracle.dot(synth.numpy_uniform(synth.SEED_X, s, ch), synth.numpy_uniform(synth.SEED_Y, s, ch))
+        ref += r
+        mag += m
+    assert_tol([got], [ref], [mag], "dot 2^31")
+
+
+# ===================================================================== GEMV
+GEMV_SHAPES = [(1, 1), (7, 3), (5, 129), (3, 5000), (300, 1000), (1000, 4), (33, 4096), (257, 8192), (4096, 4096),
+               (17, 32768)]
+
+
+@pytest.mark.parametrize("m,n", GEMV_SHAPES)
+def test_gemv_parity(cuda_device, m, n):
+    A = rand(synth.SEED_A, (m, n))
+    x = rand(synth.SEED_X, (n,))
+    got = lift.lift_gemv(dev_np(A, cuda_device), dev_np(x, cuda_device)).cpu().numpy()
+    ref, mag = oracle.gemv(A, x)
+    assert_tol(got, ref, mag, f"gemv {m}x{n}")
+
+
+def test_gemv_positive_data_8192(cuda_device):
+    m, n = 512, 8192
+    A = rand(synth.SEED_A, (m, n), "pos")
+    x = rand(synth.SEED_X, (n,), "pos")
+    got = lift.lift_gemv(dev_np(A, cuda_device), dev_np(x, cuda_device)).cpu().numpy()
+    ref, mag = oracle.gemv(A, x)
+    assert_tol(got, ref, mag, "gemv positive")
+
+
+def test_gemv_unaligned_and_ragged(cuda_device):
+    m, n = 37, 1001
+    buf = dev_np(rand(2, (m * n + 3,)), cuda_device)
+    A = buf[3:].view(m, n)  # 12-byte offset: scalar path
+    x = dev_np(rand(0, (n,)), cuda_device)
+    got = lift.lift_gemv(A, x).cpu().numpy()
+    ref, mag = oracle.gemv(A.cpu().numpy(), x.cpu().numpy())
+    assert_tol(got, ref, mag, "gemv unaligned")
+
+
+def test_gemv_empty(cuda_device):
+    A = torch.zeros(5, 0, device=cuda_device)
+    y = lift.lift_gemv(A, torch.zeros(0, device=cuda_device))
+    assert torch.equal(y, torch.zeros(5, device=cuda_device))
+    y = lift.lift_gemv(torch.zeros(0, 7, device=cuda_device), torch.zeros(7, device=cuda_device))
+    assert y.numel() == 0
+
+
+@pytest.mark.parametrize("n", [4096, 8192, 32768])
+def test_gemv_exact_structured(cuda_device, n):
+    m = 64
+    ones = torch.ones(m, n, device=cuda_device)
+    assert torch.equal(lift.lift_gemv(ones, torch.ones(n, device=cuda_device)), torch.full((m,), float(n), device=cuda_device))
+    H = dev_np(synth.hadamard(256), cuda_device)
+    for k in (0, 5, 255):
+        e = torch.zeros(256, device=cuda_device)
+        e[k] = 1
+        assert torch.equal(lift.lift_gemv(H, e), H[:, k].contiguous())
+    I = torch.eye(512, device=cuda_device)
+    x = dev_np(rand(0, (512,)), cuda_device)
+    assert torch.equal(lift.lift_gemv(I, x), x)
+
+
+def test_gemv_config_invariant_and_shard_bitwise(cuda_device):
+    """Canonical per-row order: every launch configuration and every row
+    shard gives the same bits (what makes g-GPU == 1-GPU bitwise)."""
+    m, n = 1000, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    base = lift.lift_gemv(A, x)
+    for wpr, rg in ((8, 1), (8, 2), (8, 4), (4, 2), (4, 4), (4, 8), (2, 4), (2, 8), (1, 8), (1, 16), (1, 32)):
+        for xs in (0, 1):
+            got = lift.lift_gemv_tuned(A, x, wpr=wpr, rg=rg, xsmem=xs)
+            assert torch.equal(got, base), (wpr, rg, xs)
+    got = lift.lift_gemv_tuned(A, x, blocks=3)
+    assert torch.equal(got, base)
+    for r0, r1 in ((0, 1), (0, 500), (500, 1000), (123, 877)):
+        assert torch.equal(lift.lift_gemv(A[r0:r1], x), base[r0:r1])
+
+
+def test_gemv_nan_propagates(cuda_device):
+    m, n = 16, 256
+    A = dev_np(rand(2, (m, n)), cuda_device)
+    x = dev_np(rand(0, (n,)), cuda_device)
+    x[17] = float("nan")
+    assert torch.isnan(lift.lift_gemv(A, x)).all()
+
+
+def test_gemv_nondefault_stream_and_graph(cuda_device):
+    m, n = 2048, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    ref = lift.lift_gemv(A, x)
+    s = torch.cuda.Stream()
+    with torch.cuda.stream(s):
+        y = torch.empty(m, device=cuda_device)
+        lift.lift_gemv(A, x, out=y)
+    s.synchronize()
+    assert torch.equal(y, ref)
+    g = torch.cuda.CUDAGraph()
+    y2 = torch.empty(m, device=cuda_device)
+    with torch.cuda.graph(g):
+        lift.lift_gemv(A, x, out=y2)
+    y2.zero_()
+    g.replay()
+    torch.cuda.synchronize()
+    assert torch.equal(y2, ref)
+
+
+@pytest.mark.slow
+def test_gemv_full_size_65536x32768_sampled(cuda_device):
+    """configs[4] large GEMV (8 GiB A) in the bench's launch configuration;
+    sampled rows checked against the oracle regenerated on the host."""
+    m, n = 65536, 32768
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    y = lift.lift_gemv(A, x).cpu().numpy()
+    rows = np.unique(np.concatenate([[0, 1, m - 1, m // 2], np.random.RandomState(7).randint(0, m, 60)]))
+    xs = synth.numpy_uniform(synth.SEED_X, 0, n)
+    As = np.stack([synth.numpy_matrix_rows(synth.SEED_A, n, r, r + 1)[0] for r in rows])
+    ref, mag = oracle.gemv(As, xs)
+    assert_tol(y[rows], ref, mag, "gemv 65536x32768 sampled")
+
+
+# ===================================================================== GESUMMV
+@pytest.mark.parametrize("m,n", [(1, 1), (9, 7), (100, 1000), (64, 4096), (1024, 8192), (3, 32768)])
+@pytest.mark.parametrize("ab", [(ALPHA, BETA), (-0.75, 3.0), (0.0, 1.0), (1.0, 0.0), (-1.0, -1.0)])
+def test_gesummv_parity(cuda_device, m, n, ab):
+    al, be = ab
+    A = rand(synth.SEED_A, (m, n))
+    B = rand(synth.SEED_B, (m, n))
+    x = rand(synth.SEED_X, (n,))
+    got = lift.lift_gesummv(al, dev_np(A, cuda_device), be, dev_np(B, cuda_device), dev_np(x, cuda_device))
+    ref, mag = oracle.gesummv(al, A, be, B, x)
+    assert_tol(got.cpu().numpy(), ref, mag, f"gesummv {m}x{n} {ab}")
+
+
+def test_gesummv_full_size_8192(cuda_device):
+    """configs[2] at one GPU, every row."""
+    m = n = 8192
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    B = synth.torch_matrix_rows(synth.SEED_B, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    got = lift.lift_gesummv(ALPHA, A, BETA, B, x).cpu().numpy()
+    ref, mag = oracle.gesummv(ALPHA, A.cpu().numpy(), BETA, B.cpu().numpy(), x.cpu().numpy())
+    assert_tol(got, ref, mag, "gesummv 8192")
+
+
+def test_gesummv_reductions_bitwise(cuda_device):
+    m, n = 300, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    B = synth.torch_matrix_rows(synth.SEED_B, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    g = lift.lift_gemv(A, x)
+    # same canonical row order in both kernels: beta = 0 gives alpha * gemv exactly
+    assert torch.equal(lift.lift_gesummv(ALPHA, A, 0.0, B, x), ALPHA * g)
+    assert torch.equal(lift.lift_gesummv(1.0, A, 0.0, B, x), g)
+    assert torch.equal(lift.lift_gesummv(0.0, B, 1.0, A, x), g)
+    # ones: (alpha + beta) * n exactly
+    ones = torch.ones(8, n, device=cuda_device)
+    got = lift.lift_gesummv(1.5, ones, 1.25, ones, torch.ones(n, device=cuda_device))
+    assert torch.equal(got, torch.full((8,), 2.75 * n, device=cuda_device))
+    # sharded rows bitwise
+    full = lift.lift_gesummv(ALPHA, A, BETA, B, x)
+    assert torch.equal(lift.lift_gesummv(ALPHA, A[100:200], BETA, B[100:200], x), full[100:200])
+
+
+# ===================================================================== ATAX
+ATAX_SHAPES = [(1, 1), (5, 3), (3, 7), (64, 32), (1000, 300), (300, 1001), (4096, 4096), (2000, 16384), (100, 20000)]
+
+
+@pytest.mark.parametrize("m,n", ATAX_SHAPES)
+@pytest.mark.parametrize("algo", ["auto", "fused", "twopass"])
+def test_atax_parity(cuda_device, m, n, algo):
+    A = rand(synth.SEED_A, (m, n))
+    x = rand(synth.SEED_X, (n,))
+    Ad, xd = dev_np(A, cuda_device), dev_np(x, cuda_device)
+    if algo == "fused" and n % 4 != 0 or (algo == "fused" and n > 16384):
+        with pytest.raises(lift.LiftError):
+            lift.lift_atax(Ad, xd, algo=algo)
+        return
+    got = lift.lift_atax(Ad, xd, algo=algo).cpu().numpy()
+    ref, mag = oracle.atax(A, x)
+    assert_tol(got, ref, mag, f"atax {m}x{n} {algo}")
+
+
+@pytest.mark.parametrize("algo", ["fused", "twopass"])
+def test_atax_full_size_8192(cuda_device, algo):
+    """configs[3] at one GPU, every output."""
+    m = n = 8192
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    got = lift.lift_atax(A, x, algo=algo).cpu().numpy()
+    ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+    assert_tol(got, ref, mag, f"atax 8192 {algo}")
+
+
+@pytest.mark.parametrize("algo", ["fused", "twopass"])
+def test_atax_exact_structured(cuda_device, algo):
+    n = 4096
+    H = dev_np(synth.hadamard(n), cuda_device)
+    for k in (0, 77, n - 1):
+        e = torch.zeros(n, device=cuda_device)
+        e[k] = 1
+        want = torch.zeros(n, device=cuda_device)
+        want[k] = n
+        assert torch.equal(lift.lift_atax(H, e, algo=algo), want)  # H^T H = n I
+    x = dev_np(rand(0, (1024,)), cuda_device)
+    I = torch.eye(1024, device=cuda_device)
+    assert torch.equal(lift.lift_atax(I, x, algo=algo), x)
+    perm = torch.randperm(1024, generator=torch.Generator().manual_seed(0))
+    P = I[perm].contiguous()
+    assert torch.equal(lift.lift_atax(P, x, algo=algo), x)
+
+
+def test_atax_empty(cuda_device):
+    y = lift.lift_atax(torch.zeros(0, 9, device=cuda_device), torch.ones(9, device=cuda_device))
+    assert torch.equal(y, torch.zeros(9, device=cuda_device))
+
+
+def test_atax_deterministic(cuda_device):
+    m, n = 3000, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    for algo in ("fused", "twopass"):
+        a = lift.lift_atax(A, x, algo=algo)
+        for _ in range(3):
+            assert torch.equal(lift.lift_atax(A, x, algo=algo), a)
+
+
+def test_atax_unaligned(cuda_device):
+    m, n = 50, 301
+    buf = dev_np(rand(2, (m * n + 1,)), cuda_device)
+    A = buf[1:].view(m, n)
+    x = dev_np(rand(0, (n,)), cuda_device)
+    got = lift.lift_atax(A, x).cpu().numpy()
+    ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+    assert_tol(got, ref, mag, "atax unaligned")
