@@ -7,8 +7,8 @@
  *
  *   wpr     warps cooperating on one row: 1, 2, 4 or 8 (0 = automatic)
  *   rg      rows in flight per block:  wpr*rg*32 threads per block must be
- *           one of the compiled shapes (wpr,rg) in {(8,1),(8,2),(8,4),(4,2),
- *           (4,4),(4,8),(2,4),(2,8),(1,8),(1,16),(1,32)} (0 = automatic)
+ *           one of the compiled shapes (wpr,rg) in {(8,1),(8,2),(4,2),(4,4),
+ *           (2,4),(2,8),(1,8)} (0 = automatic)
  *   blocks  grid size (0 = persistent grid sized from the SM count)
  *   xsmem   1 = stage x in shared memory with the bulk-copy engine,
  *           0 = read x through the L1 cache, -1 = automatic

@@ -208,168 +208,185 @@ cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const
 }
 
 // ---------------------------------------------------------------------------
-// fused single pass (TMA-staged rows, producer / consumer warps)
+// fused single pass (bulk-copy-staged rows)
+//
+// Stage = one row of A (n*4 bytes) in a ring of NST shared-memory slots, each
+// with a "full" mbarrier completed by the bulk-copy engine.  All 512 threads
+// consume CR rows per step: CR partial dots in flight (ILP), ONE block barrier
+// for all CR reductions, then CR rank-1 updates of the y registers.  The
+// barrier also proves every thread has copied the step's rows into registers,
+// so right after it thread 0 refills those CR slots with the rows NST ahead —
+// no producer warp and no "empty" barriers are needed, and NST - CR .. NST
+// rows are always in flight.
 // ---------------------------------------------------------------------------
-constexpr int kFusedConsumerWarps = 16;
-constexpr int kFusedConsumers = kFusedConsumerWarps * kWarp;  // 512
-constexpr int kFusedThreads = kFusedConsumers + kWarp;        // + 1 producer warp
+constexpr int kFusedWarps = 16;
+constexpr int kFusedThreads = kFusedWarps * kWarp;  // 512
 constexpr int kFusedSmemBudget = 200 * 1024;
+constexpr int kFusedMaxStages = 16;
+constexpr int64_t kFusedMinN = 256;  // below this, rows are too short to stream efficiently
 
 struct FusedPlan {
-    int qc;       // vector columns per consumer thread (1, 2, 4, 8)
-    int rb;       // rows per stage
-    int nst;      // stages
+    int qc;       // float4 columns per thread (1, 2, 4, 8)
+    int cr;       // rows per step
+    int nst;      // stages (rows) in the ring
+    size_t hdr;   // barrier + reduction header bytes
     size_t smem;  // dynamic smem bytes
 };
 
-template <int RB>
-__host__ __device__ constexpr int fused_hdr_bytes(int nst) {
-    // full[nst], empty[nst] mbarriers + red[2][RB][16] floats, 128-B aligned
-    return ((16 * nst + 2 * RB * kFusedConsumerWarps * 4) + 127) / 128 * 128;
-}
-
 static bool fused_plan(int64_t n, FusedPlan *p) {
+    if (n <= 0 || n % 4 != 0) return false;
     const int64_t nv = n / 4;
     int qc = 1;
-    while (qc < 8 && (int64_t)qc * kFusedConsumers < nv) qc *= 2;
-    if ((int64_t)qc * kFusedConsumers < nv) return false;
+    while (qc < 8 && (int64_t)qc * kFusedThreads < nv) qc *= 2;
+    if ((int64_t)qc * kFusedThreads < nv) return false;
     const size_t row = (size_t)n * 4;
-    int rb = (int)(32768 / row);
-    if (rb < 1) rb = 1;
-    if (rb > 4) rb = 4;
-    if (rb == 3) rb = 2;
-    int nst = 0;
-    size_t smem = 0;
-    for (int k = 8; k >= 2; --k) {
-        size_t hdr = (size_t)((16 * k + 2 * rb * kFusedConsumerWarps * 4) + 127) / 128 * 128;
-        size_t tot = hdr + (size_t)k * rb * row;
-        if (tot <= (size_t)kFusedSmemBudget) {
-            nst = k;
-            smem = tot;
-            break;
-        }
-    }
-    if (nst == 0) return false;
+    const size_t hdr = (size_t)((8 * kFusedMaxStages + 2 * 4 * kFusedWarps * 4) + 127) / 128 * 128;
+    int64_t nst = (int64_t)(((size_t)kFusedSmemBudget - hdr) / row);
+    if (nst > kFusedMaxStages) nst = kFusedMaxStages;
+    // rows per step: at most 4 (register budget a[cr][qc]), and small enough
+    // that >= 2 further steps of rows are already in flight (lookahead)
+    int cr = (int)(nst / 3);
+    if (cr > 4) cr = 4;
+    if (qc >= 8 && cr > 2) cr = 2;
+    if (cr == 3) cr = 2;
+    if (cr < 1) return false;
+    if (nst < cr + 1) return false;
     p->qc = qc;
-    p->rb = rb;
-    p->nst = nst;
-    p->smem = smem;
+    p->cr = cr;
+    p->nst = (int)nst;
+    p->hdr = hdr;
+    p->smem = hdr + (size_t)nst * row;
     return true;
 }
 
 bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
     FusedPlan p;
-    return aligned16 && m > 0 && n > 0 && n % 4 == 0 && fused_plan(n, &p);
+    return aligned16 && m > 0 && fused_plan(n, &p);
 }
 
-template <int QC, int RB>
+bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
+    return atax_fused_supported(m, n, aligned16) && n >= kFusedMinN;
+}
+
+template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
-    k_atax_fused(int64_t m, int64_t n, int nst, const float *__restrict__ A, const float *__restrict__ x,
+    k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
                  float *__restrict__ P) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
-    uint64_t *empty = full + nst;
-    float *red = reinterpret_cast<float *>(smem + 16 * nst);  // [2][RB][16]
-    float *stage0 = reinterpret_cast<float *>(smem + fused_hdr_bytes<RB>(nst));
+    float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
+    float *stage0 = reinterpret_cast<float *>(smem + hdr);
 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int tid = threadIdx.x;
     const int64_t nv = n / 4;
     const int64_t r0 = m * blockIdx.x / gridDim.x, r1 = m * (blockIdx.x + 1) / gridDim.x;
-    const size_t stage_floats = (size_t)RB * n;
+    const uint32_t row_bytes = (uint32_t)(n * 4);
 
-    if (threadIdx.x == 0) {
-        for (int i = 0; i < nst; ++i) {
-            mbar_init(full + i, 1);
-            mbar_init(empty + i, kFusedConsumerWarps);
-        }
+    if (tid == 0) {
+        for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         fence_mbar_init();
     }
     __syncthreads();
-
-    if (warp == kFusedConsumerWarps) {
-        // ---------------- producer: stream rows of A into the stage ring ----------------
-        if (lane == 0) {
-            int it = 0;
-            for (int64_t r = r0; r < r1; r += RB, ++it) {
-                const int st = it % nst;
-                const int use = it / nst;
-                if (use > 0) mbar_wait_parity(empty + st, (uint32_t)((use - 1) & 1));
-                const int rows = (int)((r1 - r) < RB ? (r1 - r) : RB);
-                const uint32_t bytes = (uint32_t)(rows * n * 4);
-                mbar_arrive_expect_tx(full + st, bytes);
-                float *dst = stage0 + (size_t)st * stage_floats;
-                for (int i = 0; i < rows; ++i)
-                    bulk_g2s(dst + (size_t)i * n, A + (r + i) * n, (uint32_t)(n * 4), full + st);
-            }
+    if (tid == 0) {  // prologue: fill the ring
+        for (int i = 0; i < nst && r0 + i < r1; ++i) {
+            mbar_arrive_expect_tx(full + i, row_bytes);
+            bulk_g2s(stage0 + (size_t)i * n, A + (r0 + i) * n, row_bytes, full + i);
         }
-        return;
     }
 
-    // ---------------- consumers ----------------
-    const int tid = threadIdx.x;  // 0..511
     float4 xr[QC], yr[QC];
     const float4 *x4 = reinterpret_cast<const float4 *>(x);
 #pragma unroll
     for (int q = 0; q < QC; ++q) {
-        const int64_t c = tid + (int64_t)kFusedConsumers * q;
+        const int64_t c = tid + (int64_t)kFusedThreads * q;
         xr[q] = c < nv ? ld_ro4(x4 + c) : zero4();
         yr[q] = zero4();
     }
-    int it = 0, buf = 0;
-    for (int64_t r = r0; r < r1; r += RB, ++it, buf ^= 1) {
-        const int st = it % nst;
-        const int use = it / nst;
-        const int rows = (int)((r1 - r) < RB ? (r1 - r) : RB);
-        mbar_wait_parity(full + st, (uint32_t)(use & 1));
-        const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)st * stage_floats);
-        float4 a[RB][QC];
+    int it = 0, buf = 0;  // it = rows consumed so far
+    for (int64_t r = r0; r < r1; r += CR, buf ^= 1) {
+        const int rows = (int)((r1 - r) < CR ? (r1 - r) : CR);
+        float4 a[CR][QC];
 #pragma unroll
-        for (int i = 0; i < RB; ++i)
+        for (int i = 0; i < CR; ++i) {
+            if (i < rows) {
+                const int st = (it + i) % nst;
+                mbar_wait_parity(full + st, (uint32_t)(((it + i) / nst) & 1));
+                const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)st * n);
 #pragma unroll
-            for (int q = 0; q < QC; ++q) {
-                const int64_t c = tid + (int64_t)kFusedConsumers * q;
-                a[i][q] = (i < rows && c < nv) ? S4[(int64_t)i * nv + c] : zero4();
+                for (int q = 0; q < QC; ++q) {
+                    const int64_t c = tid + (int64_t)kFusedThreads * q;
+                    a[i][q] = c < nv ? S4[c] : zero4();
+                }
+            } else {
+#pragma unroll
+                for (int q = 0; q < QC; ++q) a[i][q] = zero4();
             }
-        __syncwarp();
-        if (lane == 0) asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(empty + st)) : "memory");
-        // t_r partials: this thread's columns of row r . x
-        float *rb = red + buf * RB * kFusedConsumerWarps;
+        }
+        // partial dots of this thread's columns, CR rows at once
+        float *rb = red + buf * CR * kFusedWarps;
+        float d[CR];
 #pragma unroll
-        for (int i = 0; i < RB; ++i) {
+        for (int i = 0; i < CR; ++i) {
             float4 acc = zero4();
 #pragma unroll
             for (int q = 0; q < QC; ++q) fma4(acc, a[i][q], xr[q]);
-            const float d = warp_sum(hsum4(acc));
-            if (lane == 0) rb[i * kFusedConsumerWarps + warp] = d;
+            d[i] = hsum4(acc);
         }
-        named_bar_sync(1, kFusedConsumers);
 #pragma unroll
-        for (int i = 0; i < RB; ++i) {
+        for (int o = 16; o > 0; o >>= 1)
+#pragma unroll
+            for (int i = 0; i < CR; ++i) d[i] = __fadd_rn(d[i], __shfl_xor_sync(0xffffffffu, d[i], o));
+        if (lane == 0) {
+#pragma unroll
+            for (int i = 0; i < CR; ++i) rb[i * kFusedWarps + warp] = d[i];
+        }
+        __syncthreads();  // reductions visible AND every thread is done reading this step's slots
+        if (tid == 0) {
+            for (int i = 0; i < rows; ++i) {
+                const int64_t rn = r + i + nst;  // the row NST ahead reuses this slot
+                if (rn < r1) {
+                    const int st = (it + i) % nst;
+                    mbar_arrive_expect_tx(full + st, row_bytes);
+                    bulk_g2s(stage0 + (size_t)st * n, A + rn * n, row_bytes, full + st);
+                }
+            }
+        }
+#pragma unroll
+        for (int i = 0; i < CR; ++i) {
             if (i < rows) {
-                float v[kFusedConsumerWarps];
+                float v[kFusedWarps];
+                const float4 *rb4 = reinterpret_cast<const float4 *>(rb + i * kFusedWarps);
 #pragma unroll
-                for (int w = 0; w < kFusedConsumerWarps; ++w) v[w] = rb[i * kFusedConsumerWarps + w];
-                const float t = pair_tree<kFusedConsumerWarps>(v);  // t_r = A_r . x
+                for (int w = 0; w < kFusedWarps / 4; ++w) {
+                    const float4 t4 = rb4[w];
+                    v[4 * w] = t4.x;
+                    v[4 * w + 1] = t4.y;
+                    v[4 * w + 2] = t4.z;
+                    v[4 * w + 3] = t4.w;
+                }
+                const float t = pair_tree<kFusedWarps>(v);  // t_r = A_r . x
 #pragma unroll
                 for (int q = 0; q < QC; ++q) fma4s(yr[q], a[i][q], t);  // y += A_r^T t_r
             }
         }
+        it += rows;
     }
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
 #pragma unroll
     for (int q = 0; q < QC; ++q) {
-        const int64_t c = tid + (int64_t)kFusedConsumers * q;
+        const int64_t c = tid + (int64_t)kFusedThreads * q;
         if (c < nv) P4[c] = yr[q];
     }
 }
 
-template <int QC, int RB>
-static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m, int64_t n, const float *A,
-                             const float *x, float *P, int blocks, cudaStream_t s) {
-    auto k = k_atax_fused<QC, RB>;
+template <int QC, int CR>
+static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const float *A, const float *x, float *P,
+                             int blocks, cudaStream_t s) {
+    auto k = k_atax_fused<QC, CR>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e != cudaSuccess) return e;
-    k<<<blocks, kFusedThreads, p.smem, s>>>(m, n, p.nst, A, x, P);
+    k<<<blocks, kFusedThreads, p.smem, s>>>(m, n, p.nst, (int)p.hdr, A, x, P);
     return cudaGetLastError();
 }
 
@@ -384,12 +401,13 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     if (G > kMaxSplits) G = kMaxSplits;
     if (G > m) G = m;
     cudaError_t e = cudaErrorInvalidValue;
-#define LIFT_FUSED_CASE(QC, RB) \
-    if (p.qc == QC && p.rb == RB) e = run_fused<QC, RB>(d, p, m, n, A, x, P, (int)G, s);
-    // fused_plan pairs: nv <= 512 -> (1, 4); <= 1024 -> (2, 2); <= 2048 -> (4, 1); <= 4096 -> (8, 1)
+#define LIFT_FUSED_CASE(QC, CR) \
+    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, (int)G, s);
     LIFT_FUSED_CASE(1, 4)
-    LIFT_FUSED_CASE(2, 2)
-    LIFT_FUSED_CASE(4, 1)
+    LIFT_FUSED_CASE(2, 4)
+    LIFT_FUSED_CASE(4, 4)
+    LIFT_FUSED_CASE(4, 2)
+    LIFT_FUSED_CASE(8, 2)
     LIFT_FUSED_CASE(8, 1)
 #undef LIFT_FUSED_CASE
     if (e != cudaSuccess) return e;

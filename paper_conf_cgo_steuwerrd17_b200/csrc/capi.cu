@@ -192,7 +192,7 @@ int lift_atax_algo_run(int algo, int64_t m, int64_t n, const float *A, const flo
     DeviceInfo d;
     cudaError_t e = lift::device_info(&d);
     if (e != cudaSuccess) return cuda_status(e);
-    const bool fused = (algo == LIFT_ATAX_FUSED) || (algo == LIFT_ATAX_AUTO && fused_ok);
+    const bool fused = (algo == LIFT_ATAX_FUSED) || (algo == LIFT_ATAX_AUTO && lift::atax_fused_preferred(m, n, aligned));
     if (fused) return cuda_status(lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream));
     return cuda_status(lift::launch_atax_twopass(d, m, n, A, x, y, workspace, (cudaStream_t)stream));
 }

@@ -120,8 +120,13 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     float *partials = reinterpret_cast<float *>(static_cast<char *>(workspace) + kDotTicketBytes);
     const bool vec = ((reinterpret_cast<uintptr_t>(x) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
     const int64_t units = vec ? (n >> 2) : n;
-    // enough blocks to give every thread >= 1 unit; at most a full resident wave
-    const int per_sm = 2048 / TPB;
+    // enough blocks to give every thread >= 1 unit; at most ONE resident wave
+    // (a second partial wave would serialise half the stream)
+    int per_sm = 0;
+    cudaError_t e = vec ? cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dot<TPB, U, true>, TPB, 0)
+                        : cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dot<TPB, U, false>, TPB, 0);
+    if (e != cudaSuccess) return e;
+    if (per_sm < 1) per_sm = 1;
     int64_t want = (units + TPB - 1) / TPB;
     int64_t cap = (int64_t)d.sms * per_sm;
     if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;

@@ -28,6 +28,8 @@ namespace lift {
 
 constexpr int kSlices = 8;
 constexpr int kVLanes = kSlices * kWarp;  // 256 virtual lanes per row
+// vector loads per lane per batch (x2 in flight with the one-batch prefetch)
+constexpr int kBatchLoads = 4;
 
 template <int VEC>
 struct Vec;
@@ -75,7 +77,7 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
     using V = Vec<VEC>;
     using T = typename V::T;
     constexpr int KQ = kSlices / WPR;                                    // slices per warp
-    constexpr int UK = (8 / (KQ * NMAT)) > 0 ? (8 / (KQ * NMAT)) : 1;  // k-steps per batch
+    constexpr int UK = (kBatchLoads / (KQ * NMAT)) > 0 ? (kBatchLoads / (KQ * NMAT)) : 1;  // k-steps per batch
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 16);
@@ -94,31 +96,45 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
     }
 
     const int64_t row_step = (int64_t)gridDim.x * RG;
-    int buf = 0;
-    for (int64_t row = (int64_t)blockIdx.x * RG + g; row < m; row += row_step, buf ^= 1) {
+    int64_t row = (int64_t)blockIdx.x * RG + g;
+
+    // One continuous stream of load batches over (row, k0): batch i+1 is
+    // issued before batch i is consumed, including across the row boundary,
+    // so a warp keeps loads in flight while it reduces a finished row.
+    auto load_batch = [&](int64_t r, int64_t k0, T (&dst)[NMAT][UK][KQ]) {
+        const float *Ar = A + r * n;
+        const float *Br = (NMAT == 2) ? B + r * n : nullptr;
+#pragma unroll
+        for (int u = 0; u < UK; ++u)
+#pragma unroll
+            for (int q = 0; q < KQ; ++q) {
+                const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
+                const bool ok = (k0 + u < kcount) && (j < nv);
+#pragma unroll
+                for (int mt = 0; mt < NMAT; ++mt) dst[mt][u][q] = ok ? V::ld_stream(mt == 0 ? Ar : Br, j) : V::zero();
+            }
+    };
+
+    if (row < m) {
+        T cur[NMAT][UK][KQ];
         T acc[NMAT][KQ];
 #pragma unroll
         for (int mt = 0; mt < NMAT; ++mt)
 #pragma unroll
             for (int q = 0; q < KQ; ++q) acc[mt][q] = V::zero();
-        const float *Ar = A + row * n;
-        const float *Br = (NMAT == 2) ? B + row * n : nullptr;
-
-        for (int64_t k0 = 0; k0 < kcount; k0 += UK) {
-            T a[NMAT][UK][KQ];
-            bool ok[UK][KQ];
-#pragma unroll
-            for (int u = 0; u < UK; ++u)
-#pragma unroll
-                for (int q = 0; q < KQ; ++q) {
-                    const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
-                    ok[u][q] = (k0 + u < kcount) && (j < nv);
-#pragma unroll
-                    for (int mt = 0; mt < NMAT; ++mt)
-                        a[mt][u][q] = ok[u][q] ? V::ld_stream(mt == 0 ? Ar : Br, j) : V::zero();
-                }
+        load_batch(row, 0, cur);
+        int64_t k0 = 0;
+        int buf = 0;
+        while (true) {
+            int64_t nk = k0 + UK, nrow = row;
+            if (nk >= kcount) {
+                nk = 0;
+                nrow = row + row_step;
+            }
+            T nxt[NMAT][UK][KQ];
+            if (nrow < m) load_batch(nrow, nk, nxt);
             if constexpr (XSMEM) {
-                if (x_pending) {  // first batch: A loads are in flight, now wait for x
+                if (x_pending) {  // A loads are in flight; now wait for x
                     stage_wait(bar);
                     x_pending = false;
                 }
@@ -129,62 +145,76 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
                 for (int q = 0; q < KQ; ++q) {
                     const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
                     T xv = V::zero();
-                    if (ok[u][q]) {
+                    if ((k0 + u < kcount) && (j < nv)) {
                         if constexpr (XSMEM)
                             xv = V::ld_x(xs, j);
                         else
                             xv = V::ld_x_global(x, j);
                     }
 #pragma unroll
-                    for (int mt = 0; mt < NMAT; ++mt) V::fma(acc[mt][q], a[mt][u][q], xv);
+                    for (int mt = 0; mt < NMAT; ++mt) V::fma(acc[mt][q], cur[mt][u][q], xv);
                 }
-        }
 
-        // slice values (butterfly), then the pairwise tree over the 8 slices
-        float w[NMAT][KQ];
-#pragma unroll
-        for (int mt = 0; mt < NMAT; ++mt)
-#pragma unroll
-            for (int q = 0; q < KQ; ++q) w[mt][q] = warp_sum(V::hsum(acc[mt][q]));
-
-        float s[NMAT];
-        bool writer;
-        if constexpr (WPR == 1) {
-#pragma unroll
-            for (int mt = 0; mt < NMAT; ++mt) s[mt] = pair_tree<kSlices>(w[mt]);
-            writer = (lane == 0);
-        } else {
-            float *r = red + ((buf * RG + g) * NMAT) * kSlices;
-            if (lane == 0) {
+            if (nk == 0) {
+                // row done: slice values (butterfly), then the pairwise tree over the 8 slices
+                float w[NMAT][KQ];
 #pragma unroll
                 for (int mt = 0; mt < NMAT; ++mt)
 #pragma unroll
-                    for (int q = 0; q < KQ; ++q) r[mt * kSlices + wr * KQ + q] = w[mt][q];
-            }
-            if constexpr (RG == 1)
-                __syncthreads();
-            else
-                named_bar_sync(1 + g, WPR * kWarp);
-            writer = (wr == 0 && lane == 0);
-            if (writer) {
+                    for (int q = 0; q < KQ; ++q) {
+                        w[mt][q] = warp_sum(V::hsum(acc[mt][q]));
+                        acc[mt][q] = V::zero();
+                    }
+                float s[NMAT];
+                bool writer;
+                if constexpr (WPR == 1) {
 #pragma unroll
-                for (int mt = 0; mt < NMAT; ++mt) {
-                    float v[kSlices];
+                    for (int mt = 0; mt < NMAT; ++mt) s[mt] = pair_tree<kSlices>(w[mt]);
+                    writer = (lane == 0);
+                } else {
+                    float *r = red + ((buf * RG + g) * NMAT) * kSlices;
+                    if (lane == 0) {
 #pragma unroll
-                    for (int p = 0; p < kSlices; ++p) v[p] = r[mt * kSlices + p];
-                    s[mt] = pair_tree<kSlices>(v);
+                        for (int mt = 0; mt < NMAT; ++mt)
+#pragma unroll
+                            for (int q = 0; q < KQ; ++q) r[mt * kSlices + wr * KQ + q] = w[mt][q];
+                    }
+                    if constexpr (RG == 1)
+                        __syncthreads();
+                    else
+                        named_bar_sync(1 + g, WPR * kWarp);
+                    writer = (wr == 0 && lane == 0);
+                    if (writer) {
+#pragma unroll
+                        for (int mt = 0; mt < NMAT; ++mt) {
+                            float v[kSlices];
+#pragma unroll
+                            for (int p = 0; p < kSlices; ++p) v[p] = r[mt * kSlices + p];
+                            s[mt] = pair_tree<kSlices>(v);
+                        }
+                    }
+                    buf ^= 1;
                 }
+                if (writer) {
+                    if constexpr (NMAT == 1)
+                        y[row] = s[0];
+                    else
+                        y[row] = __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, s[1]));
+                }
+                if (nrow >= m) break;
             }
-        }
-        if (writer) {
-            if constexpr (NMAT == 1)
-                y[row] = s[0];
-            else
-                y[row] = __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, s[1]));
+            row = nrow;
+            k0 = nk;
+#pragma unroll
+            for (int mt = 0; mt < NMAT; ++mt)
+#pragma unroll
+                for (int u = 0; u < UK; ++u)
+#pragma unroll
+                    for (int q = 0; q < KQ; ++q) cur[mt][u][q] = nxt[mt][u][q];
         }
     }
     if constexpr (XSMEM) {
-        // a block that received no row must still retire its bulk copy
+        // a row group that received no row must still retire the bulk copy
         if (x_pending) stage_wait(bar);
     }
 }
@@ -225,15 +255,11 @@ static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int64_t m,
         return run_gemv<NMAT, VEC, W, R, XSMEM>(d, m, n, A, B, x, y, alpha, beta, blocks, s);
     LIFT_GEMV_CASE(8, 1)
     LIFT_GEMV_CASE(8, 2)
-    LIFT_GEMV_CASE(8, 4)
     LIFT_GEMV_CASE(4, 2)
     LIFT_GEMV_CASE(4, 4)
-    LIFT_GEMV_CASE(4, 8)
     LIFT_GEMV_CASE(2, 4)
     LIFT_GEMV_CASE(2, 8)
     LIFT_GEMV_CASE(1, 8)
-    LIFT_GEMV_CASE(1, 16)
-    LIFT_GEMV_CASE(1, 32)
 #undef LIFT_GEMV_CASE
     return cudaErrorInvalidValue;
 }
@@ -263,7 +289,11 @@ cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, con
     if (rg == 0) {
         // 256-thread blocks by default; 1024 when one block per SM holds a large x
         rg = 256 / (wpr * kWarp);
-        if (xsmem && 2 * (x_bytes + 1024) > (size_t)d.smem_per_sm) rg = 1024 / (wpr * kWarp);
+        if (xsmem && 2 * (x_bytes + 1024) > (size_t)d.smem_per_sm) {
+            // one block per SM holds the large x: 512 threads, >= 2 warps per row
+            if (wpr < 2) wpr = 2;
+            rg = 512 / (wpr * kWarp);
+        }
         if (rg < 1) rg = 1;
     }
     if (vec) {

@@ -41,6 +41,7 @@ cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, con
 size_t atax_twopass_ws_bytes(int64_t m, int64_t n);
 size_t atax_fused_ws_bytes(int64_t m, int64_t n);
 bool atax_fused_supported(int64_t m, int64_t n, bool aligned16);
+bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16);
 cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
                                 float *y, void *ws, cudaStream_t s);
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,

@@ -1,0 +1,137 @@
+"""Row sharding of the hot path across the GPUs of one node (north_star).
+
+One process per GPU; ``torch.distributed`` (backend "nccl" on GPUs) carries
+exactly ONE collective per op — the exchange step each op really has:
+
+=========  ==========================================  ======================================
+op         partition                                   collective
+=========  ==========================================  ======================================
+dot        contiguous element slices of x, y           all_reduce(SUM) of one fp32 scalar
+GEMV       contiguous row blocks of A; x replicated    all_gather_into_tensor of y blocks
+GESUMMV    row blocks of A and B;  x replicated        all_gather_into_tensor of y blocks
+ATAX       row blocks of A; x replicated               reduce(SUM, dst) (or all_reduce) of
+           (t_r = A_r x is row-local: no exchange)     the partial A_r^T (A_r x)
+=========  ==========================================  ======================================
+
+The paper evaluates one GPU only (L999-1007); this layer is new.  Reading R19:
+rank r owns rows [floor(r*m/g), floor((r+1)*m/g)).  GEMV/GESUMMV rows use a
+canonical per-row summation order (include/lift.h), so the gathered y is
+bitwise identical to the single-GPU result.
+
+The per-rank compute is the C-ABI library.  ``local`` lets tests substitute
+the per-rank compute (tests/test_shard_gloo.py runs this exact host logic on
+CPU with the gloo backend and world_size 2); the product path always uses the
+CUDA library and never falls back.
+"""
+from __future__ import annotations
+
+from dataclasses import dataclass
+from typing import Callable, Optional
+
+import torch
+import torch.distributed as dist
+
+
+def partition_rows(m: int, world: int, rank: int) -> tuple[int, int]:
+    """Rows [r0, r1) of rank `rank` out of `world` (reading R19)."""
+    if world < 1 or not (0 <= rank < world) or m < 0:
+        raise ValueError(f"bad partition request m={m} world={world} rank={rank}")
+    return (m * rank) // world, (m * (rank + 1)) // world
+
+
+def shard_sizes(m: int, world: int) -> list[int]:
+    return [partition_rows(m, world, r)[1] - partition_rows(m, world, r)[0] for r in range(world)]
+
+
+@dataclass
+class LocalOps:
+    """Per-rank compute.  Defaults are the CUDA C-ABI ops."""
+    dot: Callable
+    gemv: Callable
+    gesummv: Callable
+    atax: Callable
+
+
+def cuda_ops() -> LocalOps:
+    from . import lift_atax, lift_dot, lift_gemv, lift_gesummv
+
+    return LocalOps(
+        dot=lambda x, y, out=None: lift_dot(x, y, out=out),
+        gemv=lambda A, x, out=None: lift_gemv(A, x, out=out),
+        gesummv=lambda al, A, be, B, x, out=None: lift_gesummv(al, A, be, B, x, out=out),
+        atax=lambda A, x, out=None: lift_atax(A, x, out=out),
+    )
+
+
+_default_ops: Optional[LocalOps] = None
+
+
+def _ops(local: Optional[LocalOps]) -> LocalOps:
+    global _default_ops
+    if local is not None:
+        return local
+    if _default_ops is None:
+        _default_ops = cuda_ops()
+    return _default_ops
+
+
+def _world(group) -> tuple[int, int]:
+    return dist.get_world_size(group), dist.get_rank(group)
+
+
+def _gather_rows(y_loc: torch.Tensor, m: int, group, out: Optional[torch.Tensor]) -> torch.Tensor:
+    """All-gather row blocks of y into a full y (padding only when m % g != 0)."""
+    g, r = _world(group)
+    sizes = shard_sizes(m, g)
+    if y_loc.numel() != sizes[r]:
+        raise ValueError(f"rank {r} holds {y_loc.numel()} rows, partition says {sizes[r]}")
+    if all(s == sizes[0] for s in sizes):
+        y = out if out is not None else torch.empty(m, dtype=y_loc.dtype, device=y_loc.device)
+        dist.all_gather_into_tensor(y, y_loc, group=group)
+        return y
+    pad = max(sizes)
+    send = torch.zeros(pad, dtype=y_loc.dtype, device=y_loc.device)
+    send[: y_loc.numel()] = y_loc
+    buf = torch.empty(pad * g, dtype=y_loc.dtype, device=y_loc.device)
+    dist.all_gather_into_tensor(buf, send, group=group)
+    y = out if out is not None else torch.empty(m, dtype=y_loc.dtype, device=y_loc.device)
+    o = 0
+    for k, s in enumerate(sizes):
+        y[o:o + s] = buf[k * pad:k * pad + s]
+        o += s
+    return y
+
+
+def dot(x_loc: torch.Tensor, y_loc: torch.Tensor, group=None, local: Optional[LocalOps] = None) -> torch.Tensor:
+    """sum over ranks of dot(x_loc, y_loc): one all_reduce(SUM) of a 4-byte scalar."""
+    s = _ops(local).dot(x_loc, y_loc)
+    s = s.reshape(1)
+    dist.all_reduce(s, op=dist.ReduceOp.SUM, group=group)
+    return s.reshape(())
+
+
+def gemv(A_loc: torch.Tensor, x: torch.Tensor, m: int, group=None, local: Optional[LocalOps] = None,
+         y_loc: Optional[torch.Tensor] = None, out: Optional[torch.Tensor] = None) -> torch.Tensor:
+    """y = A x with A row-sharded (rank's rows A_loc); returns the full y on every rank."""
+    y_loc = _ops(local).gemv(A_loc, x, out=y_loc)
+    return _gather_rows(y_loc, m, group, out)
+
+
+def gesummv(alpha: float, A_loc: torch.Tensor, beta: float, B_loc: torch.Tensor, x: torch.Tensor, m: int,
+            group=None, local: Optional[LocalOps] = None, y_loc: Optional[torch.Tensor] = None,
+            out: Optional[torch.Tensor] = None) -> torch.Tensor:
+    """y = alpha A x + beta B x with A, B row-sharded; full y on every rank."""
+    y_loc = _ops(local).gesummv(alpha, A_loc, beta, B_loc, x, out=y_loc)
+    return _gather_rows(y_loc, m, group, out)
+
+
+def atax(A_loc: torch.Tensor, x: torch.Tensor, group=None, dst: int = 0, allreduce: bool = False,
+         local: Optional[LocalOps] = None, out: Optional[torch.Tensor] = None) -> Optional[torch.Tensor]:
+    """y = A^T (A x) = sum_r A_r^T (A_r x).  Result on `dst` (None elsewhere),
+    or on every rank with allreduce=True."""
+    y = _ops(local).atax(A_loc, x, out=out)
+    if allreduce:
+        dist.all_reduce(y, op=dist.ReduceOp.SUM, group=group)
+        return y
+    dist.reduce(y, dst=dst, op=dist.ReduceOp.SUM, group=group)
+    return y if dist.get_rank(group) == dst else None
