@@ -249,13 +249,18 @@ def run_reference(args) -> None:
 # ----------------------------------------------------------------------------
 # our arm
 # ----------------------------------------------------------------------------
-def load_traffic(kernel: str):
-    """ncu --set full DRAM bytes per launch of `kernel` (committed under profiles/)."""
+# ncu capture label of each op (tools/gpu_round.sh, tools/make_profiles.py)
+CAPTURE_LABEL = {"gemv_4096x4096": "gemv4096", "gesummv_8192x8192": "gesummv8192", "atax_8192x8192": "atax8192",
+                 "gemv_65536x32768": "gemv65536", "dot_2^31": "dot2p31"}
+
+
+def load_traffic(kernel: str, op_name: str):
+    """ncu --set full DRAM bytes per launch of `kernel` on `op_name`'s shape (profiles/traffic.json)."""
     p = os.path.join(ROOT, "profiles", "traffic.json")
     try:
         with open(p) as f:
             d = json.load(f)
-        return d.get(kernel, {}).get("dram_bytes_per_launch")
+        return d.get(f"{kernel}:{CAPTURE_LABEL[op_name]}", {}).get("dram_bytes_per_launch")
     except Exception:
         return None
 
@@ -404,7 +409,7 @@ def run_ours(args) -> None:
         kms = op_ms[dom]
     achieved = dom_bytes_rank / (kms * 1e-3) / 1e9
     roofline = {"bound": "hbm", "kernel": kernel, "op": dom_name, "achieved": round(achieved, 1), "peak": peak,
-                "unit": "GB/s", "frac": round(achieved / peak, 4), "traffic": load_traffic(kernel),
+                "unit": "GB/s", "frac": round(achieved / peak, 4), "traffic": load_traffic(kernel, dom_name),
                 "alg_bytes_per_launch": int(dom_bytes_rank), "launch_ms": round(kms, 4), "peak_source": peak_src}
 
     kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 2}[op] for _, op, _, _ in WORKLOAD)
