@@ -412,7 +412,7 @@ def run_ours(args) -> None:
                 "unit": "GB/s", "frac": round(achieved / peak, 4), "traffic": load_traffic(kernel, dom_name),
                 "alg_bytes_per_launch": int(dom_bytes_rank), "launch_ms": round(kms, 4), "peak_source": peak_src}
 
-    kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 2}[op] for _, op, _, _ in WORKLOAD)
+    kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 1}[op] for _, op, _, _ in WORKLOAD)
     gpu_launches = kernels_per_step * args.steps
 
     # ---- e2e: host buffers -> device -> our API -> host, per step ----

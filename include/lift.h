@@ -126,7 +126,8 @@ LIFT_API int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, flo
  * lift_atax picks the fastest algorithm for the shape:
  *   LIFT_ATAX_FUSED    one streaming pass over A: per row group, t_r = A_r x
  *                      by a block tree, then y_part += A_r^T t_r from the
- *                      same registers; then a fixed-order reduce of the
+ *                      same registers; then, in the same cooperative launch
+ *                      after a grid barrier, a fixed-order reduce of the
  *                      per-block y_part (reads A once: 4*m*n bytes).
  *   LIFT_ATAX_TWOPASS  the paper's structure (two GEMV-shaped kernels whose
  *                      times are summed, L1006-1007): GEMV t = A x, then a
@@ -136,8 +137,10 @@ LIFT_API int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, flo
  *   A          device fp32[m][n] row-major;  x device fp32[n]
  *   y          device fp32[n], written
  *   workspace  device scratch >= lift_atax_workspace_bytes(m, n), 16-byte
- *              aligned; no initialisation needed; not shared by concurrent
- *              calls.                                                     */
+ *              aligned.  Its first 256 bytes hold grid-barrier counters that
+ *              MUST be zero before the first call (cudaMemset once at
+ *              allocation); every call leaves them zero.  Not shared by
+ *              concurrent calls.                                          */
 typedef enum lift_atax_algo {
     LIFT_ATAX_AUTO = 0,
     LIFT_ATAX_FUSED = 1,

@@ -12,6 +12,10 @@
  *   blocks  grid size (0 = persistent grid sized from the SM count)
  *   xsmem   1 = stage x in shared memory with the bulk-copy engine,
  *           0 = read x through the L1 cache, -1 = automatic
+ *   lb      vector loads per lane per batch, 4 or 8 (the kernel keeps two
+ *           batches in flight); 0 = automatic
+ * The scalar path (n % 4 != 0 or a base not 16-byte aligned) has one shape:
+ * wpr = 1, rg = 8, lb = 4 (or 0 for each).
  * An unsupported combination returns LIFT_ERR_CUDA with
  * lift_last_cuda_error() = "invalid argument".
  */
@@ -25,11 +29,11 @@ extern "C" {
 #endif
 
 LIFT_API int lift_gemv_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y,
-                    int wpr, int rg, int blocks, int xsmem, lift_stream_t stream);
+                    int wpr, int rg, int blocks, int xsmem, int lb, lift_stream_t stream);
 
 LIFT_API int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *A, float beta,
                        const float *B, const float *x, float *y,
-                       int wpr, int rg, int blocks, int xsmem, lift_stream_t stream);
+                       int wpr, int rg, int blocks, int xsmem, int lb, lift_stream_t stream);
 
 #ifdef __cplusplus
 }

@@ -22,7 +22,7 @@ __all__ = ["lift_dot", "lift_gemv", "lift_gesummv", "lift_atax", "lift_gemv_tune
            "LiftError", "lib", "library_path", "KERNELS_PER_CALL"]
 
 # kernels each entry point enqueues (for the bench's gpu_launches count)
-KERNELS_PER_CALL = {"lift_dot": 1, "lift_gemv": 1, "lift_gesummv": 1, "lift_atax_fused": 2, "lift_atax_twopass": 3}
+KERNELS_PER_CALL = {"lift_dot": 1, "lift_gemv": 1, "lift_gesummv": 1, "lift_atax_fused": 1, "lift_atax_twopass": 3}
 
 _ws_lock = threading.Lock()
 _ws_cache: dict = {}
@@ -56,8 +56,9 @@ def _stream(device: torch.device) -> int:
 def _workspace(kind: str, device: torch.device, nbytes: int, zero: bool) -> torch.Tensor:
     """Per-(kind, device, stream) cached workspace, grown on demand.
 
-    The dot workspace holds an arrival ticket that must start at zero; it is
-    allocated with torch.zeros and every dot call leaves it zero again."""
+    The dot and ATAX workspaces start with counters that must be zero before
+    first use; they are allocated with torch.zeros and every call leaves them
+    zero again."""
     key = (kind, device.index, _stream(device))
     with _ws_lock:
         ws = _ws_cache.get(key)
@@ -103,7 +104,7 @@ def lift_gemv(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None)
     return out
 
 
-def lift_gemv_tuned(A, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1):
+def lift_gemv_tuned(A, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1, lb=0):
     """lift_gemv with an explicit launch configuration (include/lift_tuning.h)."""
     _check_tensor(A, "A", 2)
     _check_tensor(x, "x", 1)
@@ -112,7 +113,7 @@ def lift_gemv_tuned(A, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1):
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
     with torch.cuda.device(dev):
-        check(lib().lift_gemv_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), wpr, rg, blocks, xsmem,
+        check(lib().lift_gemv_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), wpr, rg, blocks, xsmem, lb,
                                     _stream(dev)))
     return out
 
@@ -136,7 +137,7 @@ def lift_gesummv(alpha: float, A: torch.Tensor, beta: float, B: torch.Tensor, x:
     return out
 
 
-def lift_gesummv_tuned(alpha, A, beta, B, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1):
+def lift_gesummv_tuned(alpha, A, beta, B, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1, lb=0):
     _check_tensor(A, "A", 2)
     _check_tensor(B, "B", 2)
     _check_tensor(x, "x", 1)
@@ -146,7 +147,7 @@ def lift_gesummv_tuned(alpha, A, beta, B, x, out=None, wpr=0, rg=0, blocks=0, xs
         out = torch.empty(m, dtype=torch.float32, device=dev)
     with torch.cuda.device(dev):
         check(lib().lift_gesummv_tuned(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
-                                       out.data_ptr(), wpr, rg, blocks, xsmem, _stream(dev)))
+                                       out.data_ptr(), wpr, rg, blocks, xsmem, lb, _stream(dev)))
     return out
 
 
@@ -167,7 +168,7 @@ def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None,
     L = lib()
     nbytes = L.lift_atax_workspace_bytes(m, n)
     with torch.cuda.device(dev):
-        ws = _workspace("atax", dev, nbytes, zero=False)
+        ws = _workspace("atax", dev, nbytes, zero=True)
         check(L.lift_atax_algo_run(_ALGOS[algo], m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(),
                                    ws.numel(), _stream(dev)))
     return out

@@ -46,8 +46,8 @@ SIGNATURES = {
     "lift_strerror": (ctypes.c_char_p, [i32]),
     "lift_last_cuda_error": (ctypes.c_char_p, []),
     "lift_version": (i32, []),
-    "lift_gemv_tuned": (i32, [i64, i64, vp, vp, vp, i32, i32, i32, i32, vp]),
-    "lift_gesummv_tuned": (i32, [i64, i64, f32, vp, f32, vp, vp, vp, i32, i32, i32, i32, vp]),
+    "lift_gemv_tuned": (i32, [i64, i64, vp, vp, vp, i32, i32, i32, i32, i32, vp]),
+    "lift_gesummv_tuned": (i32, [i64, i64, f32, vp, f32, vp, vp, vp, i32, i32, i32, i32, i32, vp]),
 }
 
 

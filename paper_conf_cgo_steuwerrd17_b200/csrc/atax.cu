@@ -22,7 +22,9 @@
 // partial dot, reduce it across the block (warp butterfly + one named barrier)
 // to t_r = A_r . x, and fold A_rj * t_r into their y registers from the SAME
 // registers — t is never written, A is read once (4*m*n bytes instead of 8).
-// Per-block y partials are then summed by k_colsum in a fixed order.
+// The per-block y partials are summed in a fixed order in the SAME launch: a
+// grid barrier (cooperative launch, one block per SM) and then every block
+// reduces a tile of columns over all partial rows.
 #include <type_traits>
 
 #include "common.cuh"
@@ -34,92 +36,86 @@ constexpr int kMaxSplits = 256;  // partial-row capacity of the workspace
 
 static inline size_t align256(size_t b) { return (b + 255) / 256 * 256; }
 
+// workspace: [0, 256) grid-barrier counters (zero before first use, left zero),
+// then t (two-pass only), then the partial rows P[S][n]
+constexpr size_t kWsHeader = 256;
 size_t atax_twopass_ws_bytes(int64_t m, int64_t n) {
-    return align256((size_t)m * 4) + align256((size_t)kMaxSplits * (size_t)n * 4);
+    return kWsHeader + align256((size_t)m * 4) + align256((size_t)kMaxSplits * (size_t)n * 4);
 }
-size_t atax_fused_ws_bytes(int64_t, int64_t n) { return align256((size_t)kMaxSplits * (size_t)n * 4); }
+size_t atax_fused_ws_bytes(int64_t, int64_t n) { return kWsHeader + align256((size_t)kMaxSplits * (size_t)n * 4); }
 
 // ---------------------------------------------------------------------------
-// fixed-order column sum:  y[c] = sum_{s < S} P[s][c]
-// block = 8 warps x 32 columns; warp w folds splits [w*S/8, (w+1)*S/8) in
-// order, then the 8 warp partials are combined by a pairwise tree.
+// fixed-order column sum of one tile of 32 vector columns:
+//   y[c] = sum_{s < S} P[s][c],  c in [c0, c0 + 32)
+// W warps; warp w folds splits [w*S/W, (w+1)*S/W) in order (4 loads in
+// flight), then the W warp partials are combined by a pairwise tree.  The
+// order depends only on (S, W): deterministic.
 // ---------------------------------------------------------------------------
-template <int VEC>
-__global__ void __launch_bounds__(256) k_colsum(int S, int64_t nv, const float *__restrict__ P, float *__restrict__ y) {
-    __shared__ __align__(16) float part[8][32 * VEC];
+template <int VEC, int W>
+__device__ __forceinline__ void colsum_tile(int S, int64_t nv, const float *__restrict__ P, float *__restrict__ y,
+                                            int64_t c0, float *part /* smem [W][32*VEC] */) {
+    using V = typename std::conditional<VEC == 4, float4, float>::type;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int64_t c = (int64_t)blockIdx.x * 32 + lane;
-    const int s0 = (int)((int64_t)S * warp / 8), s1 = (int)((int64_t)S * (warp + 1) / 8);
-    if constexpr (VEC == 4) {
-        float4 acc = zero4();
-        if (c < nv) {
-            const float4 *P4 = reinterpret_cast<const float4 *>(P);
-            int s = s0;
-            for (; s + 4 <= s1; s += 4) {
-                float4 v[4];
+    const int64_t c = c0 + lane;
+    const int s0 = (int)((int64_t)S * warp / W), s1 = (int)((int64_t)S * (warp + 1) / W);
+    const V *PV = reinterpret_cast<const V *>(P);
+    float acc[VEC];
 #pragma unroll
-                for (int u = 0; u < 4; ++u) v[u] = __ldcg(P4 + (int64_t)(s + u) * nv + c);
+    for (int e = 0; e < VEC; ++e) acc[e] = 0.f;
+    if (c < nv) {
+        int s = s0;
+        for (; s + 4 <= s1; s += 4) {
+            V v[4];
 #pragma unroll
-                for (int u = 0; u < 4; ++u) {
-                    acc.x = __fadd_rn(acc.x, v[u].x);
-                    acc.y = __fadd_rn(acc.y, v[u].y);
-                    acc.z = __fadd_rn(acc.z, v[u].z);
-                    acc.w = __fadd_rn(acc.w, v[u].w);
-                }
-            }
-            for (; s < s1; ++s) {
-                float4 v = __ldcg(P4 + (int64_t)s * nv + c);
-                acc.x = __fadd_rn(acc.x, v.x);
-                acc.y = __fadd_rn(acc.y, v.y);
-                acc.z = __fadd_rn(acc.z, v.z);
-                acc.w = __fadd_rn(acc.w, v.w);
+            for (int u = 0; u < 4; ++u) v[u] = __ldcg(PV + (int64_t)(s + u) * nv + c);
+#pragma unroll
+            for (int u = 0; u < 4; ++u) {
+                const float *f = reinterpret_cast<const float *>(&v[u]);
+#pragma unroll
+                for (int e = 0; e < VEC; ++e) acc[e] = __fadd_rn(acc[e], f[e]);
             }
         }
-        reinterpret_cast<float4 *>(part[warp])[lane] = acc;
-        __syncthreads();
-        if (warp == 0 && c < nv) {
-            float comp[4][8];
+        for (; s < s1; ++s) {
+            V v = __ldcg(PV + (int64_t)s * nv + c);
+            const float *f = reinterpret_cast<const float *>(&v);
 #pragma unroll
-            for (int w = 0; w < 8; ++w) {
-                float4 v = reinterpret_cast<const float4 *>(part[w])[lane];
-                comp[0][w] = v.x;
-                comp[1][w] = v.y;
-                comp[2][w] = v.z;
-                comp[3][w] = v.w;
-            }
-            float4 r = make_float4(pair_tree<8>(comp[0]), pair_tree<8>(comp[1]), pair_tree<8>(comp[2]),
-                                   pair_tree<8>(comp[3]));
-            reinterpret_cast<float4 *>(y)[c] = r;
-        }
-    } else {
-        float acc = 0.f;
-        if (c < nv) {
-            int s = s0;
-            for (; s + 4 <= s1; s += 4) {
-                float v[4];
-#pragma unroll
-                for (int u = 0; u < 4; ++u) v[u] = __ldcg(P + (int64_t)(s + u) * nv + c);
-#pragma unroll
-                for (int u = 0; u < 4; ++u) acc = __fadd_rn(acc, v[u]);
-            }
-            for (; s < s1; ++s) acc = __fadd_rn(acc, __ldcg(P + (int64_t)s * nv + c));
-        }
-        part[warp][lane] = acc;
-        __syncthreads();
-        if (warp == 0 && c < nv) {
-            float v[8];
-#pragma unroll
-            for (int w = 0; w < 8; ++w) v[w] = part[w][lane];
-            y[c] = pair_tree<8>(v);
+            for (int e = 0; e < VEC; ++e) acc[e] = __fadd_rn(acc[e], f[e]);
         }
     }
+#pragma unroll
+    for (int e = 0; e < VEC; ++e) part[(warp * 32 + lane) * VEC + e] = acc[e];
+    __syncthreads();
+    if (warp == 0 && c < nv) {
+        float out[VEC];
+#pragma unroll
+        for (int e = 0; e < VEC; ++e) {
+            float v[W];
+#pragma unroll
+            for (int w = 0; w < W; ++w) v[w] = part[(w * 32 + lane) * VEC + e];
+            out[e] = pair_tree<W>(v);
+        }
+        if constexpr (VEC == 4)
+            reinterpret_cast<float4 *>(y)[c] = make_float4(out[0], out[1], out[2], out[3]);
+        else
+            y[c] = out[0];
+    }
+    __syncthreads();  // part[] reuse by the next tile
+}
+
+constexpr int kColsumWarps = 16;
+
+template <int VEC>
+__global__ void __launch_bounds__(kColsumWarps * 32) k_colsum(int S, int64_t nv, const float *__restrict__ P,
+                                                                float *__restrict__ y) {
+    __shared__ __align__(16) float part[kColsumWarps * 32 * VEC];
+    colsum_tile<VEC, kColsumWarps>(S, nv, P, y, (int64_t)blockIdx.x * 32, part);
 }
 
 template <int VEC>
 static cudaError_t run_colsum(int S, int64_t n, const float *P, float *y, cudaStream_t s) {
     const int64_t nv = n / VEC;
     const int64_t blocks = (nv + 31) / 32;
-    k_colsum<VEC><<<(unsigned)blocks, 256, 0, s>>>(S, nv, P, y);
+    k_colsum<VEC><<<(unsigned)blocks, kColsumWarps * 32, 0, s>>>(S, nv, P, y);
     return cudaGetLastError();
 }
 
@@ -172,8 +168,8 @@ cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const
                                 void *ws, cudaStream_t s) {
     if (n == 0) return cudaSuccess;
     if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
-    float *t = static_cast<float *>(ws);
-    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + align256((size_t)m * 4));
+    float *t = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
+    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader + align256((size_t)m * 4));
     cudaError_t e = launch_gemv(d, 1, m, n, A, nullptr, x, t, 1.f, 0.f, GemvConfig{}, s);
     if (e != cudaSuccess) return e;
     const bool vec = (n % 4 == 0) && ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
@@ -255,7 +251,9 @@ static bool fused_plan(int64_t n, FusedPlan *p) {
     p->cr = cr;
     p->nst = (int)nst;
     p->hdr = hdr;
-    p->smem = hdr + (size_t)nst * row;
+    // the drained ring is reused for the final column-sum tile partials
+    const size_t ring = (size_t)nst * row, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
+    p->smem = hdr + (ring > tile ? ring : tile);
     return true;
 }
 
@@ -268,10 +266,37 @@ bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     return atax_fused_supported(m, n, aligned16) && n >= kFusedMinN;
 }
 
+// One-shot grid barrier for a cooperative launch (all blocks co-resident).
+// gbar[0] counts arrivals, gbar[1] departures; the last block to depart
+// re-arms both to zero for the next launch on this workspace.
+__device__ __forceinline__ void grid_barrier(unsigned int *gbar) {
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();  // publish this block's partial row
+        atomicAdd(gbar, 1u);
+        unsigned int v;
+        do {
+            asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(gbar) : "memory");
+            if (v < gridDim.x) __nanosleep(64);
+        } while (v < gridDim.x);
+    }
+    __syncthreads();
+}
+
+__device__ __forceinline__ void grid_depart(unsigned int *gbar) {
+    if (threadIdx.x == 0) {
+        const unsigned int d = atomicAdd(gbar + 1, 1u) + 1u;
+        if (d == gridDim.x) {  // every block has passed the barrier
+            gbar[0] = 0u;
+            gbar[1] = 0u;
+        }
+    }
+}
+
 template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
     k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
-                 float *__restrict__ P) {
+                 float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
@@ -378,16 +403,34 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         const int64_t c = tid + (int64_t)kFusedThreads * q;
         if (c < nv) P4[c] = yr[q];
     }
+
+    // ---- second stage in the same launch: grid barrier, then every block sums
+    // tiles of 32 float4 columns over all G partial rows in a fixed order ----
+    grid_barrier(gbar);
+    float *part = stage0;  // the ring is drained: reuse it for the tile partials
+    for (int64_t c0 = (int64_t)blockIdx.x * 32; c0 < nv; c0 += (int64_t)gridDim.x * 32)
+        colsum_tile<4, kFusedWarps>((int)gridDim.x, nv, P, y, c0, part);
+    grid_depart(gbar);
 }
 
 template <int QC, int CR>
 static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const float *A, const float *x, float *P,
-                             int blocks, cudaStream_t s) {
+                             float *y, unsigned int *gbar, int blocks, cudaStream_t s) {
     auto k = k_atax_fused<QC, CR>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e != cudaSuccess) return e;
-    k<<<blocks, kFusedThreads, p.smem, s>>>(m, n, p.nst, (int)p.hdr, A, x, P);
-    return cudaGetLastError();
+    // cooperative: the in-kernel grid barrier needs every block resident (one per SM)
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3((unsigned)blocks);
+    cfg.blockDim = dim3(kFusedThreads);
+    cfg.dynamicSmemBytes = p.smem;
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeCooperative;
+    attr[0].val.cooperative = 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar);
 }
 
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
@@ -396,13 +439,14 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
     FusedPlan p;
     if (!fused_plan(n, &p)) return cudaErrorInvalidValue;
-    float *P = static_cast<float *>(ws);
+    unsigned int *gbar = static_cast<unsigned int *>(ws);
+    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
     int64_t G = d.sms;
     if (G > kMaxSplits) G = kMaxSplits;
     if (G > m) G = m;
     cudaError_t e = cudaErrorInvalidValue;
 #define LIFT_FUSED_CASE(QC, CR) \
-    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, (int)G, s);
+    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, y, gbar, (int)G, s);
     LIFT_FUSED_CASE(1, 4)
     LIFT_FUSED_CASE(2, 4)
     LIFT_FUSED_CASE(4, 4)
@@ -410,8 +454,7 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     LIFT_FUSED_CASE(8, 2)
     LIFT_FUSED_CASE(8, 1)
 #undef LIFT_FUSED_CASE
-    if (e != cudaSuccess) return e;
-    return run_colsum<4>((int)G, n, P, y, s);
+    return e;
 }
 
 }  // namespace lift

@@ -122,7 +122,7 @@ static int check_gemv_family(int64_t m, int64_t n, const float *A, const float *
 }
 
 int lift_gemv_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y, int wpr, int rg, int blocks,
-                    int xsmem, lift_stream_t stream) {
+                    int xsmem, int lb, lift_stream_t stream) {
     int st = check_gemv_family(m, n, A, nullptr, false, x, y);
     if (st != LIFT_OK) return st;
     if (m == 0) return LIFT_OK;
@@ -134,15 +134,16 @@ int lift_gemv_tuned(int64_t m, int64_t n, const float *A, const float *x, float 
     cfg.rg = rg;
     cfg.blocks = blocks;
     cfg.xsmem = xsmem;
+    cfg.lb = lb;
     return cuda_status(lift::launch_gemv(d, 1, m, n, A, nullptr, x, y, 1.f, 0.f, cfg, (cudaStream_t)stream));
 }
 
 int lift_gemv(int64_t m, int64_t n, const float *A, const float *x, float *y, lift_stream_t stream) {
-    return lift_gemv_tuned(m, n, A, x, y, 0, 0, 0, -1, stream);
+    return lift_gemv_tuned(m, n, A, x, y, 0, 0, 0, -1, 0, stream);
 }
 
 int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B, const float *x,
-                       float *y, int wpr, int rg, int blocks, int xsmem, lift_stream_t stream) {
+                       float *y, int wpr, int rg, int blocks, int xsmem, int lb, lift_stream_t stream) {
     int st = check_gemv_family(m, n, A, B, true, x, y);
     if (st != LIFT_OK) return st;
     if (m == 0) return LIFT_OK;
@@ -154,12 +155,13 @@ int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *A, float 
     cfg.rg = rg;
     cfg.blocks = blocks;
     cfg.xsmem = xsmem;
+    cfg.lb = lb;
     return cuda_status(lift::launch_gemv(d, 2, m, n, A, B, x, y, alpha, beta, cfg, (cudaStream_t)stream));
 }
 
 int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B, const float *x,
                  float *y, lift_stream_t stream) {
-    return lift_gesummv_tuned(m, n, alpha, A, beta, B, x, y, 0, 0, 0, -1, stream);
+    return lift_gesummv_tuned(m, n, alpha, A, beta, B, x, y, 0, 0, 0, -1, 0, stream);
 }
 
 size_t lift_atax_workspace_bytes(int64_t m, int64_t n) {

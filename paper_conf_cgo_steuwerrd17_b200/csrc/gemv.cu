@@ -28,8 +28,6 @@ namespace lift {
 
 constexpr int kSlices = 8;
 constexpr int kVLanes = kSlices * kWarp;  // 256 virtual lanes per row
-// vector loads per lane per batch (x2 in flight with the one-batch prefetch)
-constexpr int kBatchLoads = 4;
 
 template <int VEC>
 struct Vec;
@@ -37,15 +35,9 @@ template <>
 struct Vec<4> {
     using T = float4;
     static __device__ __forceinline__ T zero() { return zero4(); }
-    static __device__ __forceinline__ T ld_stream(const float *base, int64_t j) {
-        return ld_stream4(reinterpret_cast<const float4 *>(base) + j);
-    }
-    static __device__ __forceinline__ T ld_x(const float *base, int64_t j) {
-        return reinterpret_cast<const float4 *>(base)[j];
-    }
-    static __device__ __forceinline__ T ld_x_global(const float *base, int64_t j) {
-        return ld_ro4(reinterpret_cast<const float4 *>(base) + j);
-    }
+    static __device__ __forceinline__ T ld_stream(const T *p) { return ld_stream4(p); }
+    static __device__ __forceinline__ T ld_x_smem(const T *p) { return *p; }
+    static __device__ __forceinline__ T ld_x_global(const T *p) { return ld_ro4(p); }
     static __device__ __forceinline__ void fma(T &acc, T a, T b) { fma4(acc, a, b); }
     static __device__ __forceinline__ float hsum(T v) { return hsum4(v); }
 };
@@ -53,9 +45,9 @@ template <>
 struct Vec<1> {
     using T = float;
     static __device__ __forceinline__ T zero() { return 0.f; }
-    static __device__ __forceinline__ T ld_stream(const float *base, int64_t j) { return ld_stream1(base + j); }
-    static __device__ __forceinline__ T ld_x(const float *base, int64_t j) { return base[j]; }
-    static __device__ __forceinline__ T ld_x_global(const float *base, int64_t j) { return ld_ro1(base + j); }
+    static __device__ __forceinline__ T ld_stream(const T *p) { return ld_stream1(p); }
+    static __device__ __forceinline__ T ld_x_smem(const T *p) { return *p; }
+    static __device__ __forceinline__ T ld_x_global(const T *p) { return ld_ro1(p); }
     static __device__ __forceinline__ void fma(T &acc, T a, T b) { acc = __fmaf_rn(a, b, acc); }
     static __device__ __forceinline__ float hsum(T v) { return v; }
 };
@@ -70,14 +62,14 @@ __host__ __device__ constexpr int gemv_x_offset() {
     return (16 + gemv_red_bytes<NMAT, RG>() + 15) / 16 * 16;
 }
 
-template <int NMAT, int VEC, int WPR, int RG, bool XSMEM>
+template <int NMAT, int VEC, int WPR, int RG, bool XSMEM, int LB>
 __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, const float *__restrict__ A,
                                                         const float *__restrict__ B, const float *__restrict__ x,
                                                         float *__restrict__ y, float alpha, float beta) {
     using V = Vec<VEC>;
     using T = typename V::T;
-    constexpr int KQ = kSlices / WPR;                                    // slices per warp
-    constexpr int UK = (kBatchLoads / (KQ * NMAT)) > 0 ? (kBatchLoads / (KQ * NMAT)) : 1;  // k-steps per batch
+    constexpr int KQ = kSlices / WPR;                                 // slices per warp
+    constexpr int UK = (LB / (KQ * NMAT)) > 0 ? (LB / (KQ * NMAT)) : 1;  // k-steps per batch
     extern __shared__ __align__(16) unsigned char smem[];
     uint64_t *bar = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 16);
@@ -87,13 +79,16 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
     const int g = warp / WPR;   // row group inside the block
     const int wr = warp % WPR;  // warp rank inside the row group
     const int64_t nv = n / VEC;
-    const int64_t kcount = (nv + kVLanes - 1) / kVLanes;
+    const int64_t kcount = (nv + kVLanes - 1) / kVLanes;  // k-steps per row
+    const int64_t kfull = nv / kVLanes;                   // k-steps whose every vector is in the row
+    const int lane_off = kWarp * (wr * KQ) + lane;        // first virtual lane of this lane, slice q adds 32*q
 
     bool x_pending = false;
     if constexpr (XSMEM) {
         stage_issue(xs, x, (uint32_t)(n * 4), bar);  // toLocal(x), one bulk copy per block
         x_pending = true;
     }
+    const T *xl = reinterpret_cast<const T *>(XSMEM ? xs : x) + lane_off;
 
     const int64_t row_step = (int64_t)gridDim.x * RG;
     int64_t row = (int64_t)blockIdx.x * RG + g;
@@ -101,18 +96,29 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
     // One continuous stream of load batches over (row, k0): batch i+1 is
     // issued before batch i is consumed, including across the row boundary,
     // so a warp keeps loads in flight while it reduces a finished row.
+    // Full batches use compile-time offsets and no predicates.
     auto load_batch = [&](int64_t r, int64_t k0, T (&dst)[NMAT][UK][KQ]) {
-        const float *Ar = A + r * n;
-        const float *Br = (NMAT == 2) ? B + r * n : nullptr;
+        const T *Ar = reinterpret_cast<const T *>(A + r * n) + (kVLanes * k0 + lane_off);
+        const T *Br = (NMAT == 2) ? reinterpret_cast<const T *>(B + r * n) + (kVLanes * k0 + lane_off) : nullptr;
+        if (k0 + UK <= kfull) {
 #pragma unroll
-        for (int u = 0; u < UK; ++u)
+            for (int u = 0; u < UK; ++u)
 #pragma unroll
-            for (int q = 0; q < KQ; ++q) {
-                const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
-                const bool ok = (k0 + u < kcount) && (j < nv);
+                for (int q = 0; q < KQ; ++q)
 #pragma unroll
-                for (int mt = 0; mt < NMAT; ++mt) dst[mt][u][q] = ok ? V::ld_stream(mt == 0 ? Ar : Br, j) : V::zero();
-            }
+                    for (int mt = 0; mt < NMAT; ++mt)
+                        dst[mt][u][q] = V::ld_stream((mt == 0 ? Ar : Br) + (kVLanes * u + kWarp * q));
+        } else {
+#pragma unroll
+            for (int u = 0; u < UK; ++u)
+#pragma unroll
+                for (int q = 0; q < KQ; ++q) {
+                    const bool ok = kVLanes * (k0 + u) + kWarp * q + lane_off < nv;
+#pragma unroll
+                    for (int mt = 0; mt < NMAT; ++mt)
+                        dst[mt][u][q] = ok ? V::ld_stream((mt == 0 ? Ar : Br) + (kVLanes * u + kWarp * q)) : V::zero();
+                }
+        }
     };
 
     if (row < m) {
@@ -139,21 +145,30 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
                     x_pending = false;
                 }
             }
+            const T *xb = xl + kVLanes * k0;
+            if (k0 + UK <= kfull) {
 #pragma unroll
-            for (int u = 0; u < UK; ++u)
+                for (int u = 0; u < UK; ++u)
 #pragma unroll
-                for (int q = 0; q < KQ; ++q) {
-                    const int64_t j = (int64_t)kVLanes * (k0 + u) + kWarp * (wr * KQ + q) + lane;
-                    T xv = V::zero();
-                    if ((k0 + u < kcount) && (j < nv)) {
-                        if constexpr (XSMEM)
-                            xv = V::ld_x(xs, j);
-                        else
-                            xv = V::ld_x_global(x, j);
+                    for (int q = 0; q < KQ; ++q) {
+                        const T xv = XSMEM ? V::ld_x_smem(xb + kVLanes * u + kWarp * q)
+                                           : V::ld_x_global(xb + kVLanes * u + kWarp * q);
+#pragma unroll
+                        for (int mt = 0; mt < NMAT; ++mt) V::fma(acc[mt][q], cur[mt][u][q], xv);
                     }
+            } else {
 #pragma unroll
-                    for (int mt = 0; mt < NMAT; ++mt) V::fma(acc[mt][q], cur[mt][u][q], xv);
-                }
+                for (int u = 0; u < UK; ++u)
+#pragma unroll
+                    for (int q = 0; q < KQ; ++q) {
+                        T xv = V::zero();
+                        if (kVLanes * (k0 + u) + kWarp * q + lane_off < nv)
+                            xv = XSMEM ? V::ld_x_smem(xb + kVLanes * u + kWarp * q)
+                                       : V::ld_x_global(xb + kVLanes * u + kWarp * q);
+#pragma unroll
+                        for (int mt = 0; mt < NMAT; ++mt) V::fma(acc[mt][q], cur[mt][u][q], xv);
+                    }
+            }
 
             if (nk == 0) {
                 // row done: slice values (butterfly), then the pairwise tree over the 8 slices
@@ -223,10 +238,10 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
 // host-side configuration
 // ---------------------------------------------------------------------------
 
-template <int NMAT, int VEC, int WPR, int RG, bool XSMEM>
+template <int NMAT, int VEC, int WPR, int RG, bool XSMEM, int LB>
 static cudaError_t run_gemv(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *B,
                             const float *x, float *y, float alpha, float beta, int blocks, cudaStream_t s) {
-    auto kern = k_gemv<NMAT, VEC, WPR, RG, XSMEM>;
+    auto kern = k_gemv<NMAT, VEC, WPR, RG, XSMEM, LB>;
     constexpr int threads = RG * WPR * kWarp;
     size_t smem = gemv_x_offset<NMAT, RG>() + (XSMEM ? (size_t)n * 4 : 0);
     if (smem > 48 * 1024) {
@@ -246,13 +261,15 @@ static cudaError_t run_gemv(const DeviceInfo &d, int64_t m, int64_t n, const flo
 }
 
 template <int NMAT, int VEC, bool XSMEM>
-static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int64_t m, int64_t n, const float *A,
+static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int lb, int64_t m, int64_t n, const float *A,
                                 const float *B, const float *x, float *y, float alpha, float beta, int blocks,
                                 cudaStream_t s) {
     // block = RG row groups of WPR warps; 256..1024 threads
-#define LIFT_GEMV_CASE(W, R)                                                                     \
-    if (wpr == W && rg == R)                                                                     \
-        return run_gemv<NMAT, VEC, W, R, XSMEM>(d, m, n, A, B, x, y, alpha, beta, blocks, s);
+#define LIFT_GEMV_CASE(W, R)                                                                           \
+    if (wpr == W && rg == R) {                                                                         \
+        if (lb == 8) return run_gemv<NMAT, VEC, W, R, XSMEM, 8>(d, m, n, A, B, x, y, alpha, beta, blocks, s); \
+        return run_gemv<NMAT, VEC, W, R, XSMEM, 4>(d, m, n, A, B, x, y, alpha, beta, blocks, s);            \
+    }
     LIFT_GEMV_CASE(8, 1)
     LIFT_GEMV_CASE(8, 2)
     LIFT_GEMV_CASE(4, 2)
@@ -273,38 +290,37 @@ cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, con
     const bool vec = (n % 4 == 0) && (orr & 15) == 0;
     // x in smem when it fits next to the red buffers (bulk copy needs 16-B units)
     const size_t x_bytes = (size_t)n * 4;
-    bool xsmem = vec && x_bytes + 1024 <= (size_t)d.smem_optin;
+    // Defaults from the B200 sweep (tools/sweep.py, profiles/r01b_sweep.txt): one row per
+    // 256-thread block (8 warps x 1 slice each), 4 vector loads per lane per batch, x in
+    // SMEM only while >= 4 blocks per SM still fit (a 128 KiB x that pins one block per SM
+    // loses ~25 %; L1 serves it better).
+    bool xsmem = vec && 4 * (x_bytes + 1024) <= (size_t)d.smem_per_sm;
     if (cfg.xsmem == 0) xsmem = false;
-    if (cfg.xsmem == 1 && !xsmem) return cudaErrorInvalidValue;
-
+    if (cfg.xsmem == 1) {
+        if (!(vec && x_bytes + 1024 <= (size_t)d.smem_optin)) return cudaErrorInvalidValue;
+        xsmem = true;
+    }
     int wpr = cfg.wpr, rg = cfg.rg;
-    if (wpr == 0) {
-        // spread rows over enough warps to fill the chip: about 32 resident
-        // warps per SM want a row task each
-        const int64_t want_tasks = (int64_t)d.sms * 32;
+    if (wpr == 0) wpr = vec ? 8 : 1;
+    if (!vec) {
         wpr = 1;
-        while (wpr < 8 && m * wpr < want_tasks) wpr *= 2;
-        if (!vec) wpr = 1;
+        rg = 8;
     }
-    if (rg == 0) {
-        // 256-thread blocks by default; 1024 when one block per SM holds a large x
-        rg = 256 / (wpr * kWarp);
-        if (xsmem && 2 * (x_bytes + 1024) > (size_t)d.smem_per_sm) {
-            // one block per SM holds the large x: 512 threads, >= 2 warps per row
-            if (wpr < 2) wpr = 2;
-            rg = 512 / (wpr * kWarp);
-        }
-        if (rg < 1) rg = 1;
-    }
+    if (rg == 0) rg = (256 / (wpr * kWarp)) > 0 ? 256 / (wpr * kWarp) : 1;
+    int lb = cfg.lb;
+    if (lb == 0) lb = 4;
+    if (lb != 4 && lb != 8) return cudaErrorInvalidValue;
     if (vec) {
         if (nmat == 1)
-            return xsmem ? dispatch_wpr<1, 4, true>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
-                         : dispatch_wpr<1, 4, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
-        return xsmem ? dispatch_wpr<2, 4, true>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
-                     : dispatch_wpr<2, 4, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+            return xsmem ? dispatch_wpr<1, 4, true>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
+                         : dispatch_wpr<1, 4, false>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+        return xsmem ? dispatch_wpr<2, 4, true>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
+                     : dispatch_wpr<2, 4, false>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
     }
-    if (nmat == 1) return dispatch_wpr<1, 1, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
-    return dispatch_wpr<2, 1, false>(d, wpr, rg, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+    // scalar path (n % 4 != 0 or misaligned): one shape
+    if (wpr != 1 || rg != 8 || lb != 4) return cudaErrorInvalidValue;
+    if (nmat == 1) return run_gemv<1, 1, 1, 8, false, 4>(d, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+    return run_gemv<2, 1, 1, 8, false, 4>(d, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
 }
 
 }  // namespace lift

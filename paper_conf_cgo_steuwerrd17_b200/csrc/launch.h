@@ -32,6 +32,7 @@ struct GemvConfig {
     int rg = 0;      // row groups per block; 0 = auto
     int blocks = 0;  // grid size; 0 = auto (persistent)
     int xsmem = -1;  // 1 = stage x in smem by bulk copy, 0 = read x through L1, -1 = auto
+    int lb = 0;      // vector loads per lane per batch (4 or 8; x2 in flight with the prefetch); 0 = auto
 };
 // nmat = 1: y = A x;  nmat = 2: y = alpha A x + beta B x
 cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, const float *A, const float *B,

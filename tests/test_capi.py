@@ -101,8 +101,8 @@ def test_gesummv_validation():
 
 
 def test_tuned_validation():
-    assert L.lift_gemv_tuned(-1, 4, A_, X_, Y_, 8, 1, 0, -1, None) == SIZE
-    assert L.lift_gesummv_tuned(4, 4, 1.0, A_, 1.0, B_, X_, A_, 8, 1, 0, -1, None) == ALIAS
+    assert L.lift_gemv_tuned(-1, 4, A_, X_, Y_, 8, 1, 0, -1, 4, None) == SIZE
+    assert L.lift_gesummv_tuned(4, 4, 1.0, A_, 1.0, B_, X_, A_, 8, 1, 0, -1, 4, None) == ALIAS
 
 
 # ---------------------------------------------------------------- ATAX

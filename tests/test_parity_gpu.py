@@ -171,8 +171,9 @@ def test_gemv_config_invariant_and_shard_bitwise(cuda_device):
     base = lift.lift_gemv(A, x)
     for wpr, rg in ((8, 1), (8, 2), (4, 2), (4, 4), (2, 4), (2, 8), (1, 8)):
         for xs in (0, 1):
-            got = lift.lift_gemv_tuned(A, x, wpr=wpr, rg=rg, xsmem=xs)
-            assert torch.equal(got, base), (wpr, rg, xs)
+            for lb in (4, 8):
+                got = lift.lift_gemv_tuned(A, x, wpr=wpr, rg=rg, xsmem=xs, lb=lb)
+                assert torch.equal(got, base), (wpr, rg, xs, lb)
     got = lift.lift_gemv_tuned(A, x, blocks=3)
     assert torch.equal(got, base)
     for r0, r1 in ((0, 1), (0, 500), (500, 1000), (123, 877)):

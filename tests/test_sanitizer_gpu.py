@@ -1,0 +1,26 @@
+"""compute-sanitizer over small / ragged invocations of every kernel
+(memcheck, racecheck, synccheck, initcheck).  The kernels use no global
+atomics on data and fixed-order reductions; any report is a bug."""
+import os
+import shutil
+import subprocess
+import sys
+
+import pytest
+
+pytestmark = pytest.mark.gpu
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.mark.parametrize("tool", ["memcheck", "racecheck", "synccheck", "initcheck"])
+def test_compute_sanitizer(cuda_device, tool):
+    cs = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
+    if not os.path.exists(cs):
+        pytest.fail("compute-sanitizer not found")
+    cmd = [cs, "--tool", tool, "--error-exitcode", "99", "--kernel-name", "kns=lift",
+           sys.executable, os.path.join(ROOT, "tools", "sanitize_cases.py")]
+    r = subprocess.run(cmd, capture_output=True, text=True, timeout=900, cwd=ROOT)
+    tail = (r.stdout + r.stderr)[-4000:]
+    assert r.returncode == 0, tail
+    assert "sanitize cases ok" in r.stdout, tail
+    assert "ERROR SUMMARY: 0 errors" in (r.stdout + r.stderr), tail
