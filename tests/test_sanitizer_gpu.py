@@ -2,6 +2,7 @@
 (memcheck, racecheck, synccheck, initcheck).  The kernels use no global
 atomics on data and fixed-order reductions; any report is a bug."""
 import os
+import re
 import shutil
 import subprocess
 import sys
@@ -17,10 +18,14 @@ def test_compute_sanitizer(cuda_device, tool):
     cs = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
     if not os.path.exists(cs):
         pytest.fail("compute-sanitizer not found")
-    cmd = [cs, "--tool", tool, "--error-exitcode", "99", "--kernel-name", "kns=lift",
+    # initcheck must see the writes of torch's fill kernels (torch.zeros workspaces), so
+    # it instruments every kernel; the other tools check only this library's kernels
+    filt = [] if tool == "initcheck" else ["--kernel-name", "kns=lift"]
+    cmd = [cs, "--tool", tool, "--error-exitcode", "99", *filt,
            sys.executable, os.path.join(ROOT, "tools", "sanitize_cases.py")]
     r = subprocess.run(cmd, capture_output=True, text=True, timeout=900, cwd=ROOT)
     tail = (r.stdout + r.stderr)[-4000:]
     assert r.returncode == 0, tail
     assert "sanitize cases ok" in r.stdout, tail
-    assert "ERROR SUMMARY: 0 errors" in (r.stdout + r.stderr), tail
+    out = r.stdout + r.stderr
+    assert re.search(r"ERROR SUMMARY: 0 errors|SUMMARY: 0 hazards displayed \(0 errors", out), tail
