@@ -155,6 +155,39 @@ LIFT_API int lift_atax_algo_run(int algo, int64_t m, int64_t n, const float *A,
                        size_t workspace_bytes, lift_stream_t stream);
 
 /* ---------------------------------------------------------------------- */
+/* Listing 1 in the paper's exact order (bitwise reproducible semantics)   */
+/* ---------------------------------------------------------------------- */
+/* partialDot (Listing 1; generated kernel Fig. 7):
+ * work group k reduces the 128-element chunk k of zip(x, y): local thread l
+ * (of 64) folds elements 2l, 2l+1 with multAndSumUp from 0, then iterate6
+ * halves 64 -> 1 with out[l] = (0 + in[2l]) + in[2l+1].  Every fp32 operation
+ * happens in exactly this order, so the result is a fixed bit pattern for
+ * given inputs (pinned against oracle/ bit for bit).
+ *
+ *   n         elements (>= 0); z gets n/128 values (Fig. 7 forms only N/128
+ *             work groups, L954; a ragged tail is ignored, as in the paper)
+ *   x, y      device fp32[n], 4-byte aligned (16-byte alignment is faster)
+ *   z         device fp32[n/128], written
+ *   contract  1: multAndSumUp = fma(x, y, a) (one rounding);
+ *             0: a + (x*y) with the product rounded first (reading R2)    */
+LIFT_API int lift_partial_dot(int64_t n, const float *x, const float *y, float *z,
+                              int contract, lift_stream_t stream);
+
+/* The whole dot in the paper's structure (reading R26): Listing 1 over
+ * ceil(n/128) zero-padded chunks, then the same work-group program with add
+ * (the second kernel the paper omits, L422-426) applied again — iterate,
+ * L312-318 — until one value remains: ceil(log128 n) launches.  Bitwise
+ * equal to oracle_dot_listing1_f32.  n == 0 writes 0.
+ *
+ *   result     device fp32[1], written
+ *   workspace  device scratch >= lift_dot_listing1_workspace_bytes(n),
+ *              16-byte aligned, no initialisation needed                 */
+LIFT_API size_t lift_dot_listing1_workspace_bytes(int64_t n);
+LIFT_API int lift_dot_listing1(int64_t n, const float *x, const float *y, float *result,
+                               void *workspace, size_t workspace_bytes, int contract,
+                               lift_stream_t stream);
+
+/* ---------------------------------------------------------------------- */
 /* library info                                                            */
 /* ---------------------------------------------------------------------- */
 LIFT_API const char *lift_strerror(int status);      /* static string, never NULL   */

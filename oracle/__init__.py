@@ -59,6 +59,8 @@ def _load():
         lib.oracle_partial_dot.argtypes = [i64, i64, f32p, f32p, f64p, f64p]
         lib.oracle_partial_dot_listing1_f32.restype = None
         lib.oracle_partial_dot_listing1_f32.argtypes = [i64, f32p, f32p, f32p, ctypes.c_int]
+        lib.oracle_dot_listing1_f32.restype = ctypes.c_float
+        lib.oracle_dot_listing1_f32.argtypes = [i64, f32p, f32p, ctypes.c_int]
         lib.oracle_version.restype = ctypes.c_int
         _lib = lib
     return _lib
@@ -145,6 +147,13 @@ def partial_dot_listing1_f32(x, y, use_fma: bool = True) -> np.ndarray:
     z = np.empty(x.size // 128, np.float32)
     _load().oracle_partial_dot_listing1_f32(x.size, _p32(x), _p32(y), _p32(z), int(bool(use_fma)))
     return z
+
+
+def dot_listing1_f32(x, y, use_fma: bool = True) -> float:
+    """The whole dot in Listing 1's structure and order, fp32 (reading R26)."""
+    x, y = _f32(x).ravel(), _f32(y).ravel()
+    assert x.shape == y.shape
+    return float(np.float32(_load().oracle_dot_listing1_f32(x.size, _p32(x), _p32(y), int(bool(use_fma)))))
 
 
 def within_tol(got, ref, mag, rtol: float = RTOL, atol: float = ATOL):

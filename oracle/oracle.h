@@ -69,6 +69,12 @@ void oracle_partial_dot(int64_t n, int64_t chunk, const float *x,
 void oracle_partial_dot_listing1_f32(int64_t n, const float *x, const float *y,
                                      float *z, int use_fma);
 
+/* The whole dot in the paper's structure (reading R26): Listing 1 over
+   ceil(n/128) zero-padded chunks, then the same work-group program with add
+   (the omitted second kernel, L422-426) applied repeatedly — iterate,
+   L312-318 — until one value remains.  fp32, paper order. */
+float oracle_dot_listing1_f32(int64_t n, const float *x, const float *y, int use_fma);
+
 int oracle_version(void);
 
 #ifdef __cplusplus

@@ -19,6 +19,7 @@ from ._lib import (LIFT_ATAX_AUTO, LIFT_ATAX_FUSED, LIFT_ATAX_TWOPASS, LiftError
                    check, lib, library_path)
 
 __all__ = ["lift_dot", "lift_gemv", "lift_gesummv", "lift_atax", "lift_gemv_tuned", "lift_gesummv_tuned",
+           "lift_partial_dot", "lift_dot_listing1",
            "LiftError", "lib", "library_path", "KERNELS_PER_CALL"]
 
 # kernels each entry point enqueues (for the bench's gpu_launches count)
@@ -171,4 +172,40 @@ def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None,
         ws = _workspace("atax", dev, nbytes, zero=True)
         check(L.lift_atax_algo_run(_ALGOS[algo], m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(),
                                    ws.numel(), _stream(dev)))
+    return out
+
+
+def lift_partial_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None = None,
+                     contract: bool = True) -> torch.Tensor:
+    """Listing 1 (L391-401) in the paper's exact order: z[k] for k < n//128."""
+    _check_tensor(x, "x", 1)
+    _check_tensor(y, "y", 1)
+    dev = _same_device(x, y)
+    if x.numel() != y.numel():
+        raise ValueError("x and y must have the same length")
+    n = x.numel()
+    if out is None:
+        out = torch.empty(n // 128, dtype=torch.float32, device=dev)
+    _check_tensor(out, "out", 1)
+    with torch.cuda.device(dev):
+        check(lib().lift_partial_dot(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), int(bool(contract)), _stream(dev)))
+    return out
+
+
+def lift_dot_listing1(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None = None,
+                      contract: bool = True) -> torch.Tensor:
+    """The whole dot in Listing 1's structure, iterated to one value (reading R26)."""
+    _check_tensor(x, "x", 1)
+    _check_tensor(y, "y", 1)
+    dev = _same_device(x, y)
+    if x.numel() != y.numel():
+        raise ValueError("x and y must have the same length")
+    if out is None:
+        out = torch.empty((), dtype=torch.float32, device=dev)
+    L = lib()
+    n = x.numel()
+    with torch.cuda.device(dev):
+        ws = _workspace("listing1", dev, L.lift_dot_listing1_workspace_bytes(n), zero=False)
+        check(L.lift_dot_listing1(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
+                                  int(bool(contract)), _stream(dev)))
     return out

@@ -17,7 +17,7 @@ CSRC = os.path.join(PKG, "csrc")
 INCLUDE = os.path.join(ROOT, "include")
 BUILD = os.path.join(PKG, "_build")
 SO = os.path.join(PKG, "liblift.so")
-UNITS = ["capi.cu", "dot.cu", "gemv.cu", "atax.cu"]
+UNITS = ["capi.cu", "dot.cu", "gemv.cu", "atax.cu", "listing1.cu"]
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 NVCC_FLAGS = ARCH + ["-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC,-fvisibility=hidden",
                      "-I", INCLUDE, "-I", CSRC, "--expt-relaxed-constexpr"]

@@ -204,6 +204,47 @@ int lift_atax(int64_t m, int64_t n, const float *A, const float *x, float *y, vo
     return lift_atax_algo_run(LIFT_ATAX_AUTO, m, n, A, x, y, workspace, workspace_bytes, stream);
 }
 
+int lift_partial_dot(int64_t n, const float *x, const float *y, float *z, int contract, lift_stream_t stream) {
+    if (!size_ok(n, 1)) return LIFT_ERR_BAD_SIZE;
+    if (contract != 0 && contract != 1) return LIFT_ERR_BAD_SIZE;
+    const int64_t groups = n / 128;
+    if (groups == 0) return LIFT_OK;
+    if (x == nullptr || y == nullptr || z == nullptr) return LIFT_ERR_NULL_PTR;
+    if (mis4(x) || mis4(y) || mis4(z)) return LIFT_ERR_MISALIGNED;
+    const Range rz = rng(z, (uint64_t)groups * 4);
+    if (overlap(rz, rng(x, (uint64_t)n * 4)) || overlap(rz, rng(y, (uint64_t)n * 4))) return LIFT_ERR_ALIAS;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    return cuda_status(lift::launch_partial_dot(d, n, x, y, z, contract == 1, (cudaStream_t)stream));
+}
+
+size_t lift_dot_listing1_workspace_bytes(int64_t n) {
+    if (!size_ok(n, 1)) return 0;
+    return lift::dot_listing1_ws_bytes(n);
+}
+
+int lift_dot_listing1(int64_t n, const float *x, const float *y, float *result, void *workspace,
+                      size_t workspace_bytes, int contract, lift_stream_t stream) {
+    if (!size_ok(n, 1)) return LIFT_ERR_BAD_SIZE;
+    if (contract != 0 && contract != 1) return LIFT_ERR_BAD_SIZE;
+    if (result == nullptr) return LIFT_ERR_NULL_PTR;
+    if (n > 0 && (x == nullptr || y == nullptr)) return LIFT_ERR_NULL_PTR;
+    if (mis4(result) || (n > 0 && (mis4(x) || mis4(y)))) return LIFT_ERR_MISALIGNED;
+    if (workspace == nullptr || workspace_bytes < lift::dot_listing1_ws_bytes(n) ||
+        (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const Range rr = rng(result, 4), rw = rng(workspace, workspace_bytes);
+    const Range rx = rng(x, (uint64_t)n * 4), ry = rng(y, (uint64_t)n * 4);
+    if (overlap(rr, rx) || overlap(rr, ry) || overlap(rr, rw) || overlap(rw, rx) || overlap(rw, ry))
+        return LIFT_ERR_ALIAS;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    return cuda_status(
+        lift::launch_dot_listing1(d, n, x, y, result, workspace, contract == 1, (cudaStream_t)stream));
+}
+
 const char *lift_strerror(int status) {
     switch (status) {
         case LIFT_OK: return "LIFT_OK: success";

@@ -48,4 +48,11 @@ cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
                               float *y, void *ws, cudaStream_t s);
 
+// ---- Listing 1 in the paper's exact order (NEXT-3) ------------------------------
+cudaError_t launch_partial_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *z, bool fma,
+                               cudaStream_t s);
+size_t dot_listing1_ws_bytes(int64_t n);
+cudaError_t launch_dot_listing1(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
+                                void *ws, bool fma, cudaStream_t s);
+
 }  // namespace lift

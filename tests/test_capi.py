@@ -159,3 +159,17 @@ def test_ctypes_signatures_match_header_arity():
         params = [p for p in m.group(1).split(",") if p.strip() and p.strip() != "void"]
         assert len(params) == len(args), (name, params)
     assert ctypes.sizeof(ctypes.c_size_t) == 8
+
+
+def test_listing1_validation():
+    assert L.lift_partial_dot(-1, X_, Y_, Y_ + (1 << 24), 1, None) == SIZE
+    assert L.lift_partial_dot(256, X_, Y_, P * 300, 2, None) == SIZE  # contract must be 0 or 1
+    assert L.lift_partial_dot(100, None, None, None, 1, None) == OK  # no work group: nothing to do
+    assert L.lift_partial_dot(256, None, Y_, P * 300, 1, None) == NULL
+    assert L.lift_partial_dot(256, X_ + 1, Y_, P * 300, 1, None) == MIS
+    assert L.lift_partial_dot(256, X_, Y_, X_ + 4, 1, None) == ALIAS
+    ws = L.lift_dot_listing1_workspace_bytes(1000)
+    assert ws >= 2 * 8 * 4
+    assert L.lift_dot_listing1(1000, X_, Y_, P * 300, W_, ws - 1, 1, None) == WS
+    assert L.lift_dot_listing1(1000, X_, Y_, W_ + 8, W_, ws, 1, None) == ALIAS
+    assert L.lift_dot_listing1(1000, X_, Y_, None, W_, ws, 1, None) == NULL

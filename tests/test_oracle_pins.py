@@ -394,3 +394,48 @@ def test_within_tol_semantics():
     assert not ok
     ok, _ = oracle.within_tol([float("nan")], [1.0], [1.0])
     assert not ok
+
+
+# ---------------------------------------------------------------------------
+# the whole dot in Listing 1's structure (reading R26)
+# ---------------------------------------------------------------------------
+
+@pytest.mark.parametrize("use_fma", [True, False])
+def test_dot_listing1_multistage_hand_derived(use_fma):
+    case = golden("listing1_fp32_order.json")["multistage_cases"][0]
+    x = np.zeros(case["n"], np.float32)
+    for k, v in case["x"].items():
+        x[int(k)] = v
+    y = np.full(case["n"], case["y_all"], np.float32)
+    assert oracle.dot_listing1_f32(x, y, use_fma) == case["expected"]
+
+
+@pytest.mark.parametrize("n", [1, 5, 127, 128, 129, 128 * 128, 128 * 128 + 7, 3 * 128 * 128 * 2 + 1])
+def test_dot_listing1_integer_exact(n):
+    x = synth.small_ints(71, n, 3)
+    y = synth.small_ints(72, n, 3)
+    ref = int((x.astype(np.int64) * y.astype(np.int64)).sum())
+    for fma in (True, False):
+        assert oracle.dot_listing1_f32(x, y, fma) == float(ref)
+
+
+def test_dot_listing1_single_group_is_partial_dot():
+    x = rand_f32(0, (128,))
+    y = rand_f32(1, (128,))
+    for fma in (True, False):
+        assert oracle.dot_listing1_f32(x, y, fma) == float(oracle.partial_dot_listing1_f32(x, y, fma)[0])
+    # n < 128: the zero-padded single chunk
+    xs, ys = x[:77], y[:77]
+    xp, yp = np.zeros(128, np.float32), np.zeros(128, np.float32)
+    xp[:77], yp[:77] = xs, ys
+    assert oracle.dot_listing1_f32(xs, ys) == float(oracle.partial_dot_listing1_f32(xp, yp)[0])
+
+
+def test_dot_listing1_close_to_fp64_and_empty():
+    assert oracle.dot_listing1_f32(np.zeros(0, np.float32), np.zeros(0, np.float32)) == 0.0
+    n = 1 << 20
+    x = rand_f32(0, (n,))
+    y = rand_f32(1, (n,))
+    s64, mag = oracle.dot(x, y)
+    # depth: 2 pair folds + 6 tree levels per stage, 3 stages at 2^20
+    assert abs(oracle.dot_listing1_f32(x, y) - s64) <= 24 * 2.0 ** -24 * mag

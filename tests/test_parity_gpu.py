@@ -338,3 +338,65 @@ def test_atax_unaligned(cuda_device):
     got = lift.lift_atax(A, x).cpu().numpy()
     ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
     assert_tol(got, ref, mag, "atax unaligned")
+
+
+# ===================================================================== Listing 1, bit for bit (NEXT-3)
+@pytest.mark.parametrize("n", [128, 256, 128 * 37, 1 << 16, (1 << 20) + 77])
+@pytest.mark.parametrize("contract", [True, False])
+def test_partial_dot_listing1_bitwise(cuda_device, n, contract):
+    x = rand(synth.SEED_X, (n,))
+    y = rand(synth.SEED_Y, (n,))
+    got = lift.lift_partial_dot(dev_np(x, cuda_device), dev_np(y, cuda_device), contract=contract).cpu().numpy()
+    ref = oracle.partial_dot_listing1_f32(x, y, use_fma=contract)
+    assert got.shape == ref.shape
+    assert np.array_equal(got.view(np.uint32), ref.view(np.uint32))
+    # and the plain-definition tolerance against fp64
+    z64, mag = oracle.partial_dot(x, y)
+    assert_tol(got, z64, mag, "partialDot vs fp64")
+
+
+@pytest.mark.parametrize("n", [0, 1, 127, 128, 129, 128 * 128, 128 * 128 + 1, (1 << 22) + 3, 3 * (1 << 21)])
+@pytest.mark.parametrize("contract", [True, False])
+def test_dot_listing1_bitwise(cuda_device, n, contract):
+    x = rand(synth.SEED_X, (n,))
+    y = rand(synth.SEED_Y, (n,))
+    got = lift.lift_dot_listing1(dev_np(x, cuda_device), dev_np(y, cuda_device), contract=contract).item()
+    ref = oracle.dot_listing1_f32(x, y, use_fma=contract)
+    assert np.float32(got).view(np.uint32) == np.float32(ref).view(np.uint32), (got, ref)
+    s64, mag = oracle.dot(x, y)
+    assert_tol([got], [s64], [mag], "dot_listing1 vs fp64")
+
+
+def test_partial_dot_listing1_golden_cases(cuda_device):
+    from conftest import golden
+
+    g = golden("listing1_fp32_order.json")
+    for case in g["cases"]:
+        x = np.zeros(128, np.float32)
+        y = np.zeros(128, np.float32)
+        for k, v in case["x"].items():
+            x[int(k)] = v
+        if "y_all" in case:
+            y[:] = case["y_all"]
+        else:
+            for k, v in case["y"].items():
+                y[int(k)] = v
+        for contract, key in ((True, "expected_fma"), (False, "expected_nofma")):
+            z = lift.lift_partial_dot(dev_np(x, cuda_device), dev_np(y, cuda_device), contract=contract)
+            assert float(z.item()) == case[key], (case["name"], contract)
+    mc = g["multistage_cases"][0]
+    x = np.zeros(mc["n"], np.float32)
+    for k, v in mc["x"].items():
+        x[int(k)] = v
+    y = np.full(mc["n"], mc["y_all"], np.float32)
+    assert lift.lift_dot_listing1(dev_np(x, cuda_device), dev_np(y, cuda_device)).item() == mc["expected"]
+
+
+def test_partial_dot_unaligned(cuda_device):
+    n = 128 * 50 + 3
+    xb = dev_np(rand(0, (n + 1,)), cuda_device)
+    yb = dev_np(rand(1, (n + 2,)), cuda_device)
+    x, y = xb[1:], yb[2:]
+    got = lift.lift_partial_dot(x, y).cpu().numpy()
+    ref = oracle.partial_dot_listing1_f32(x.cpu().numpy(), y.cpu().numpy())
+    assert np.array_equal(got.view(np.uint32), ref.view(np.uint32))
