@@ -155,6 +155,31 @@ LIFT_API int lift_atax_algo_run(int algo, int64_t m, int64_t n, const float *A,
                        size_t workspace_bytes, lift_stream_t stream);
 
 /* ---------------------------------------------------------------------- */
+/* BLAS-complete GEMV (CLBlast SGEMV contract)                             */
+/* ---------------------------------------------------------------------- */
+/* Table 1's GEMV reference is CLBlast (L1030), whose SGEMV computes
+ *     y = alpha * op(A) * x + beta * y,   op(A) = A (trans = 0) or A^T (trans = 1)
+ * A is m x n with leading dimension lda:
+ *     layout = 0 (row-major):    element (i, j) at A[i*lda + j], lda >= n
+ *     layout = 1 (column-major): element (i, j) at A[i + j*lda], lda >= m
+ * trans = 0: x in R^n, y in R^m;  trans = 1: x in R^m, y in R^n.
+ * beta == 0: y is not read (BLAS convention: NaN/garbage in y is ignored).
+ * A column-major matrix is the row-major transpose, so (layout 1, trans t)
+ * runs the (layout 0, trans !t) kernels.  Non-transposed rows use the GEMV
+ * kernel (canonical per-row order; alpha = 1, beta = 0 is bitwise lift_gemv);
+ * transposed ones the column-blocked pass of two-pass ATAX + a fixed-order
+ * column sum, with the epilogue y = alpha*s + beta*y (products rounded, then
+ * one rounded add).
+ *
+ *   workspace  needed only for the transposed-row path:
+ *              >= lift_sgemv_workspace_bytes(layout, trans, m, n) bytes,
+ *              16-byte aligned (may be NULL when that is 0)             */
+LIFT_API size_t lift_sgemv_workspace_bytes(int layout, int trans, int64_t m, int64_t n);
+LIFT_API int lift_sgemv(int layout, int trans, int64_t m, int64_t n, float alpha,
+                        const float *A, int64_t lda, const float *x, float beta, float *y,
+                        void *workspace, size_t workspace_bytes, lift_stream_t stream);
+
+/* ---------------------------------------------------------------------- */
 /* Listing 1 in the paper's exact order (bitwise reproducible semantics)   */
 /* ---------------------------------------------------------------------- */
 /* partialDot (Listing 1; generated kernel Fig. 7):

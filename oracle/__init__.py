@@ -61,6 +61,9 @@ def _load():
         lib.oracle_partial_dot_listing1_f32.argtypes = [i64, f32p, f32p, f32p, ctypes.c_int]
         lib.oracle_dot_listing1_f32.restype = ctypes.c_float
         lib.oracle_dot_listing1_f32.argtypes = [i64, f32p, f32p, ctypes.c_int]
+        lib.oracle_sgemv.restype = None
+        lib.oracle_sgemv.argtypes = [ctypes.c_int, ctypes.c_int, i64, i64, ctypes.c_float, f32p, i64, f32p,
+                                     ctypes.c_float, f32p, f64p, f64p]
         lib.oracle_version.restype = ctypes.c_int
         _lib = lib
     return _lib
@@ -154,6 +157,19 @@ def dot_listing1_f32(x, y, use_fma: bool = True) -> float:
     x, y = _f32(x).ravel(), _f32(y).ravel()
     assert x.shape == y.shape
     return float(np.float32(_load().oracle_dot_listing1_f32(x.size, _p32(x), _p32(y), int(bool(use_fma)))))
+
+
+def sgemv(layout, trans, m, n, alpha, A_buf, lda, x, beta, y_in=None):
+    """(y, mag): BLAS SGEMV on the stored buffer A_buf (flat fp32), see oracle.h."""
+    A_buf = _f32(A_buf).ravel()
+    x = _f32(x).ravel()
+    ylen = n if trans else m
+    yi = _f32(y_in).ravel() if y_in is not None else np.zeros(ylen, np.float32)
+    y = np.empty(ylen, np.float64)
+    mag = np.empty(ylen, np.float64)
+    _load().oracle_sgemv(int(layout), int(trans), m, n, ctypes.c_float(alpha), _p32(A_buf), lda, _p32(x),
+                         ctypes.c_float(beta), _p32(yi), _p64(y), _p64(mag))
+    return y, mag
 
 
 def within_tol(got, ref, mag, rtol: float = RTOL, atol: float = ATOL):

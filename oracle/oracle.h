@@ -75,6 +75,12 @@ void oracle_partial_dot_listing1_f32(int64_t n, const float *x, const float *y,
    L312-318 — until one value remains.  fp32, paper order. */
 float oracle_dot_listing1_f32(int64_t n, const float *x, const float *y, int use_fma);
 
+/* BLAS SGEMV (CLBlast contract, Table 1; NEXT-4):
+   y = alpha*op(A) x + beta*y_in; layout 0 row-major A[i*lda+j], 1 column-major
+   A[i+j*lda]; op = A (trans 0) or A^T (trans 1); beta == 0 does not read y_in. */
+void oracle_sgemv(int layout, int trans, int64_t m, int64_t n, float alpha, const float *A, int64_t lda,
+                  const float *x, float beta, const float *y_in, double *y, double *mag);
+
 int oracle_version(void);
 
 #ifdef __cplusplus

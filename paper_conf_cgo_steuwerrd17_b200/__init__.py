@@ -19,7 +19,7 @@ from ._lib import (LIFT_ATAX_AUTO, LIFT_ATAX_FUSED, LIFT_ATAX_TWOPASS, LiftError
                    check, lib, library_path)
 
 __all__ = ["lift_dot", "lift_gemv", "lift_gesummv", "lift_atax", "lift_gemv_tuned", "lift_gesummv_tuned",
-           "lift_partial_dot", "lift_dot_listing1",
+           "lift_partial_dot", "lift_dot_listing1", "lift_sgemv",
            "LiftError", "lib", "library_path", "KERNELS_PER_CALL"]
 
 # kernels each entry point enqueues (for the bench's gpu_launches count)
@@ -209,3 +209,38 @@ def lift_dot_listing1(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None
         check(L.lift_dot_listing1(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
                                   int(bool(contract)), _stream(dev)))
     return out
+
+
+def lift_sgemv(alpha: float, A: torch.Tensor, x: torch.Tensor, beta: float = 0.0, y: torch.Tensor | None = None,
+               trans: bool = False, layout: str = "row", lda: int | None = None, shape=None) -> torch.Tensor:
+    """BLAS SGEMV: y = alpha * op(A) x + beta * y (CLBlast contract, NEXT-4).
+
+    A is the stored buffer: a 2-D tensor whose rows are the matrix's rows
+    (layout="row") or columns (layout="col"), possibly wider than the matrix
+    (lda = A.shape[1] unless given).  `shape` = (m, n) of the logical matrix
+    (default: from A).  y is updated in place when given (beta != 0 reads it).
+    """
+    _check_tensor(A, "A", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, x)
+    lay = {"row": 0, "col": 1}[layout]
+    if shape is None:
+        shape = tuple(A.shape) if lay == 0 else (A.shape[1], A.shape[0])
+    m, n = shape
+    ld = A.shape[1] if lda is None else lda
+    ylen = n if trans else m
+    if y is None:
+        if beta != 0.0:
+            raise ValueError("beta != 0 needs y")
+        y = torch.empty(ylen, dtype=torch.float32, device=dev)
+    _check_tensor(y, "y", 1)
+    if y.numel() != ylen or x.numel() != (m if trans else n):
+        raise ValueError("x / y length does not match op(A)")
+    L = lib()
+    need = L.lift_sgemv_workspace_bytes(lay, int(bool(trans)), m, n)
+    with torch.cuda.device(dev):
+        ws = _workspace("sgemv", dev, need, zero=True) if need else None
+        check(L.lift_sgemv(lay, int(bool(trans)), m, n, float(alpha), A.data_ptr(), ld, x.data_ptr(), float(beta),
+                           y.data_ptr(), ws.data_ptr() if ws is not None else None, ws.numel() if ws is not None else 0,
+                           _stream(dev)))
+    return y

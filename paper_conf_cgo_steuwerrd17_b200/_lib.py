@@ -43,6 +43,8 @@ SIGNATURES = {
     "lift_atax_workspace_bytes": (sz, [i64, i64]),
     "lift_atax": (i32, [i64, i64, vp, vp, vp, vp, sz, vp]),
     "lift_atax_algo_run": (i32, [i32, i64, i64, vp, vp, vp, vp, sz, vp]),
+    "lift_sgemv_workspace_bytes": (sz, [i32, i32, i64, i64]),
+    "lift_sgemv": (i32, [i32, i32, i64, i64, f32, vp, i64, vp, f32, vp, vp, sz, vp]),
     "lift_partial_dot": (i32, [i64, vp, vp, vp, i32, vp]),
     "lift_dot_listing1_workspace_bytes": (sz, [i64]),
     "lift_dot_listing1": (i32, [i64, vp, vp, vp, vp, sz, i32, vp]),

@@ -53,7 +53,8 @@ size_t atax_fused_ws_bytes(int64_t, int64_t n) { return kWsHeader + align256((si
 // ---------------------------------------------------------------------------
 template <int VEC, int W>
 __device__ __forceinline__ void colsum_tile(int S, int64_t nv, const float *__restrict__ P, float *__restrict__ y,
-                                            int64_t c0, float *part /* smem [W][32*VEC] */) {
+                                            int64_t c0, float *part /* smem [W][32*VEC] */, float alpha = 1.f,
+                                            float beta = 0.f, bool axpby = false) {
     using V = typename std::conditional<VEC == 4, float4, float>::type;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int64_t c = c0 + lane;
@@ -93,6 +94,9 @@ __device__ __forceinline__ void colsum_tile(int S, int64_t nv, const float *__re
 #pragma unroll
             for (int w = 0; w < W; ++w) v[w] = part[(w * 32 + lane) * VEC + e];
             out[e] = pair_tree<W>(v);
+            if (axpby)  // y = alpha*sum + beta*y, y not read when beta == 0 (BLAS)
+                out[e] = beta == 0.f ? __fmul_rn(alpha, out[e])
+                                     : __fadd_rn(__fmul_rn(alpha, out[e]), __fmul_rn(beta, y[c * VEC + e]));
         }
         if constexpr (VEC == 4)
             reinterpret_cast<float4 *>(y)[c] = make_float4(out[0], out[1], out[2], out[3]);
@@ -106,16 +110,18 @@ constexpr int kColsumWarps = 16;
 
 template <int VEC>
 __global__ void __launch_bounds__(kColsumWarps * 32) k_colsum(int S, int64_t nv, const float *__restrict__ P,
-                                                                float *__restrict__ y) {
+                                                                float *__restrict__ y, float alpha, float beta,
+                                                                bool axpby) {
     __shared__ __align__(16) float part[kColsumWarps * 32 * VEC];
-    colsum_tile<VEC, kColsumWarps>(S, nv, P, y, (int64_t)blockIdx.x * 32, part);
+    colsum_tile<VEC, kColsumWarps>(S, nv, P, y, (int64_t)blockIdx.x * 32, part, alpha, beta, axpby);
 }
 
 template <int VEC>
-static cudaError_t run_colsum(int S, int64_t n, const float *P, float *y, cudaStream_t s) {
+static cudaError_t run_colsum(int S, int64_t n, const float *P, float *y, cudaStream_t s, float alpha = 1.f,
+                              float beta = 0.f, bool axpby = false) {
     const int64_t nv = n / VEC;
     const int64_t blocks = (nv + 31) / 32;
-    k_colsum<VEC><<<(unsigned)blocks, kColsumWarps * 32, 0, s>>>(S, nv, P, y);
+    k_colsum<VEC><<<(unsigned)blocks, kColsumWarps * 32, 0, s>>>(S, nv, P, y, alpha, beta, axpby);
     return cudaGetLastError();
 }
 
@@ -123,8 +129,9 @@ static cudaError_t run_colsum(int S, int64_t n, const float *P, float *y, cudaSt
 // two-pass, pass 2: partials[s][j] = sum_{i in split s} A_ij t_i
 // ---------------------------------------------------------------------------
 template <int VEC, int TPB, int UR>
-__global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int S, const float *__restrict__ A,
-                                                   const float *__restrict__ t, float *__restrict__ P) {
+__global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int64_t lda, int S,
+                                                   const float *__restrict__ A, const float *__restrict__ t,
+                                                   float *__restrict__ P) {
     extern __shared__ float ts[];  // t for this row split (toLocal)
     using V = typename std::conditional<VEC == 4, float4, float>::type;
     const int s = blockIdx.y;
@@ -134,6 +141,7 @@ __global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int S, 
     const int64_t nv = n / VEC;
     const int64_t c = (int64_t)blockIdx.x * TPB + threadIdx.x;
     if (c >= nv) return;
+    const int64_t ldv = lda / VEC;  // row stride in vectors
     const V *A4 = reinterpret_cast<const V *>(A);
     V acc;
     if constexpr (VEC == 4) acc = zero4(); else acc = 0.f;
@@ -143,9 +151,9 @@ __global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int S, 
 #pragma unroll
         for (int u = 0; u < UR; ++u) {
             if constexpr (VEC == 4)
-                a[u] = ld_stream4(A4 + (r + u) * nv + c);
+                a[u] = ld_stream4(A4 + (r + u) * ldv + c);
             else
-                a[u] = ld_stream1(A + (r + u) * n + c);
+                a[u] = ld_stream1(A + (r + u) * lda + c);
         }
 #pragma unroll
         for (int u = 0; u < UR; ++u) {
@@ -157,22 +165,18 @@ __global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int S, 
     }
     for (; r < r1; ++r) {
         if constexpr (VEC == 4)
-            fma4s(acc, ld_stream4(A4 + r * nv + c), ts[r - r0]);
+            fma4s(acc, ld_stream4(A4 + r * ldv + c), ts[r - r0]);
         else
-            acc = __fmaf_rn(ld_stream1(A + r * n + c), ts[r - r0], acc);
+            acc = __fmaf_rn(ld_stream1(A + r * lda + c), ts[r - r0], acc);
     }
     reinterpret_cast<V *>(P)[(int64_t)s * nv + c] = acc;
 }
 
-cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
-                                void *ws, cudaStream_t s) {
-    if (n == 0) return cudaSuccess;
-    if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
-    float *t = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
-    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader + align256((size_t)m * 4));
-    cudaError_t e = launch_gemv(d, 1, m, n, A, nullptr, x, t, 1.f, 0.f, GemvConfig{}, s);
-    if (e != cudaSuccess) return e;
-    const bool vec = (n % 4 == 0) && ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
+// partials[s][j] = sum_{i in split s} A_ij t_i, then y = colsum (with epilogue)
+static cudaError_t column_pass(const DeviceInfo &d, int64_t m, int64_t n, int64_t lda, const float *A, const float *t,
+                               float *P, float *y, float alpha, float beta, bool axpby, cudaStream_t s) {
+    const bool vec = (n % 4 == 0) && (lda % 4 == 0) &&
+                     ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
     constexpr int TPB = 256;
     const int64_t nv = vec ? n / 4 : n;
     const int64_t cblocks = (nv + TPB - 1) / TPB;
@@ -183,24 +187,64 @@ cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const
     if (S < 1) S = 1;
     const size_t smem = (size_t)((m + S - 1) / S + 1) * 4;
     dim3 grid((unsigned)cblocks, (unsigned)S);
+    cudaError_t e;
     if (vec) {
         auto k = k_atax_cols<4, TPB, 8>;
         if (smem > 48 * 1024) {
             e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
             if (e != cudaSuccess) return e;
         }
-        k<<<grid, TPB, smem, s>>>(m, n, (int)S, A, t, P);
+        k<<<grid, TPB, smem, s>>>(m, n, lda, (int)S, A, t, P);
     } else {
         auto k = k_atax_cols<1, TPB, 8>;
         if (smem > 48 * 1024) {
             e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
             if (e != cudaSuccess) return e;
         }
-        k<<<grid, TPB, smem, s>>>(m, n, (int)S, A, t, P);
+        k<<<grid, TPB, smem, s>>>(m, n, lda, (int)S, A, t, P);
     }
     e = cudaGetLastError();
     if (e != cudaSuccess) return e;
-    return vec ? run_colsum<4>((int)S, n, P, y, s) : run_colsum<1>((int)S, n, P, y, s);
+    return vec ? run_colsum<4>((int)S, n, P, y, s, alpha, beta, axpby)
+               : run_colsum<1>((int)S, n, P, y, s, alpha, beta, axpby);
+}
+
+cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
+                                void *ws, cudaStream_t s) {
+    if (n == 0) return cudaSuccess;
+    if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
+    float *t = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
+    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader + align256((size_t)m * 4));
+    GemvArgs g;
+    g.m = m;
+    g.n = n;
+    g.lda = n;
+    g.A = A;
+    g.x = x;
+    g.y = t;
+    cudaError_t e = launch_gemv(d, g, GemvConfig{}, s);  // pass 1: t = A x
+    if (e != cudaSuccess) return e;
+    return column_pass(d, m, n, n, A, t, P, y, 1.f, 0.f, false, s);  // pass 2: y = A^T t
+}
+
+size_t gemv_t_ws_bytes(int64_t, int64_t n) { return kWsHeader + align256((size_t)kMaxSplits * (size_t)n * 4); }
+
+cudaError_t launch_gemv_t(const DeviceInfo &d, int64_t m, int64_t n, int64_t lda, float alpha, const float *A,
+                          const float *x, float beta, float *y, void *ws, cudaStream_t s) {
+    if (n == 0) return cudaSuccess;
+    if (m == 0) {  // y = beta * y (y not read when beta == 0)
+        GemvArgs g;  // a 0-column GEMV over the n entries of y applies exactly that epilogue
+        g.m = n;
+        g.n = 0;
+        g.lda = 0;
+        g.y = y;
+        g.alpha = alpha;
+        g.beta = beta;
+        g.epi = kEpiAxpby;
+        return launch_gemv(d, g, GemvConfig{}, s);
+    }
+    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
+    return column_pass(d, m, n, lda, A, x, P, y, alpha, beta, true, s);
 }
 
 // ---------------------------------------------------------------------------
@@ -243,7 +287,8 @@ static bool fused_plan(int64_t n, FusedPlan *p) {
     // that >= 2 further steps of rows are already in flight (lookahead)
     int cr = (int)(nst / 3);
     if (cr > 4) cr = 4;
-    if (qc >= 8 && cr > 2) cr = 2;
+    if (qc >= 4 && cr > 2) cr = 2;  // two steps of a[cr][qc] live in registers (software pipeline)
+    if (qc >= 8) cr = 1;
     if (cr == 3) cr = 2;
     if (cr < 1) return false;
     if (nst < cr + 1) return false;
@@ -264,6 +309,62 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
 
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     return atax_fused_supported(m, n, aligned16) && n >= kFusedMinN;
+}
+
+// Fixed-order column sum of the vector columns [c0, c1) over S partial rows,
+// by one 512-thread block: 16 columns per pass, 32 row splits per column
+// (each thread folds ~S/32 rows in order, all loads in flight), then the 32
+// split sums of a column are combined by a pairwise tree.  Deterministic:
+// the order depends only on S.
+__device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__restrict__ P, float *__restrict__ y,
+                                             int64_t c0, int64_t c1, float4 *part /* smem [32][16] */) {
+    constexpr int CW = 16, SPL = 32;
+    const int tid = threadIdx.x;
+    const int col = tid % CW, sp = tid / CW;
+    const int s0 = (int)((int64_t)S * sp / SPL), s1 = (int)((int64_t)S * (sp + 1) / SPL);
+    const float4 *P4 = reinterpret_cast<const float4 *>(P);
+    for (int64_t cb = c0; cb < c1; cb += CW) {
+        const int64_t c = cb + col;
+        float4 acc = zero4();
+        if (c < c1) {
+            int s = s0;
+            for (; s + 8 <= s1; s += 8) {
+                float4 v[8];
+#pragma unroll
+                for (int u = 0; u < 8; ++u) v[u] = __ldcg(P4 + (int64_t)(s + u) * nv + c);
+#pragma unroll
+                for (int u = 0; u < 8; ++u) {
+                    acc.x = __fadd_rn(acc.x, v[u].x);
+                    acc.y = __fadd_rn(acc.y, v[u].y);
+                    acc.z = __fadd_rn(acc.z, v[u].z);
+                    acc.w = __fadd_rn(acc.w, v[u].w);
+                }
+            }
+            for (; s < s1; ++s) {
+                const float4 v = __ldcg(P4 + (int64_t)s * nv + c);
+                acc.x = __fadd_rn(acc.x, v.x);
+                acc.y = __fadd_rn(acc.y, v.y);
+                acc.z = __fadd_rn(acc.z, v.z);
+                acc.w = __fadd_rn(acc.w, v.w);
+            }
+        }
+        part[sp * CW + col] = acc;
+        __syncthreads();
+        if (tid < CW && c < c1) {
+            float comp[4][SPL];
+#pragma unroll
+            for (int k = 0; k < SPL; ++k) {
+                const float4 v = part[k * CW + tid];
+                comp[0][k] = v.x;
+                comp[1][k] = v.y;
+                comp[2][k] = v.z;
+                comp[3][k] = v.w;
+            }
+            reinterpret_cast<float4 *>(y)[c] = make_float4(pair_tree<SPL>(comp[0]), pair_tree<SPL>(comp[1]),
+                                                           pair_tree<SPL>(comp[2]), pair_tree<SPL>(comp[3]));
+        }
+        __syncthreads();
+    }
 }
 
 // One-shot grid barrier for a cooperative launch (all blocks co-resident).
@@ -328,73 +429,98 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         xr[q] = c < nv ? ld_ro4(x4 + c) : zero4();
         yr[q] = zero4();
     }
-    int it = 0, buf = 0;  // it = rows consumed so far
-    for (int64_t r = r0; r < r1; r += CR, buf ^= 1) {
-        const int rows = (int)((r1 - r) < CR ? (r1 - r) : CR);
-        float4 a[CR][QC];
+    // Software-pipelined over steps: iteration k loads step k's rows and
+    // publishes their partial dots, then applies the rank-1 updates of step
+    // k-1 (whose block reductions are complete).  The one block barrier per
+    // iteration sits at its top, where it also proves that the previous
+    // step's slots have been read into registers, so they are refilled there.
+    int it = 0, buf = 0;   // it = rows loaded so far
+    int prow = 0;          // rows of the previous step (0: none)
+    int64_t prev_r = r0;   // first row of the previous step
+    float4 ap[CR][QC];     // the previous step's rows, kept for its rank-1 updates
 #pragma unroll
-        for (int i = 0; i < CR; ++i) {
-            if (i < rows) {
-                const int st = (it + i) % nst;
-                mbar_wait_parity(full + st, (uint32_t)(((it + i) / nst) & 1));
-                const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)st * n);
+    for (int i = 0; i < CR; ++i)
 #pragma unroll
-                for (int q = 0; q < QC; ++q) {
-                    const int64_t c = tid + (int64_t)kFusedThreads * q;
-                    a[i][q] = c < nv ? S4[c] : zero4();
-                }
-            } else {
-#pragma unroll
-                for (int q = 0; q < QC; ++q) a[i][q] = zero4();
-            }
-        }
-        // partial dots of this thread's columns, CR rows at once
-        float *rb = red + buf * CR * kFusedWarps;
-        float d[CR];
-#pragma unroll
-        for (int i = 0; i < CR; ++i) {
-            float4 acc = zero4();
-#pragma unroll
-            for (int q = 0; q < QC; ++q) fma4(acc, a[i][q], xr[q]);
-            d[i] = hsum4(acc);
-        }
-#pragma unroll
-        for (int o = 16; o > 0; o >>= 1)
-#pragma unroll
-            for (int i = 0; i < CR; ++i) d[i] = __fadd_rn(d[i], __shfl_xor_sync(0xffffffffu, d[i], o));
-        if (lane == 0) {
-#pragma unroll
-            for (int i = 0; i < CR; ++i) rb[i * kFusedWarps + warp] = d[i];
-        }
-        __syncthreads();  // reductions visible AND every thread is done reading this step's slots
+        for (int q = 0; q < QC; ++q) ap[i][q] = zero4();
+    for (int64_t r = r0;; r += CR, buf ^= 1) {
+        const int rows = r < r1 ? (int)((r1 - r) < CR ? (r1 - r) : CR) : 0;
+        __syncthreads();  // previous step: partials published, slots consumed
         if (tid == 0) {
-            for (int i = 0; i < rows; ++i) {
-                const int64_t rn = r + i + nst;  // the row NST ahead reuses this slot
+            for (int i = 0; i < prow; ++i) {
+                const int64_t rn = prev_r + i + nst;  // the row NST ahead reuses this slot
                 if (rn < r1) {
-                    const int st = (it + i) % nst;
+                    const int st = (it - prow + i) % nst;
                     mbar_arrive_expect_tx(full + st, row_bytes);
                     bulk_g2s(stage0 + (size_t)st * n, A + rn * n, row_bytes, full + st);
                 }
             }
         }
+        float4 a[CR][QC];
+        float *rb = red + buf * CR * kFusedWarps;
+        if (rows > 0) {
 #pragma unroll
-        for (int i = 0; i < CR; ++i) {
-            if (i < rows) {
-                float v[kFusedWarps];
-                const float4 *rb4 = reinterpret_cast<const float4 *>(rb + i * kFusedWarps);
+            for (int i = 0; i < CR; ++i) {
+                if (i < rows) {
+                    const int st = (it + i) % nst;
+                    mbar_wait_parity(full + st, (uint32_t)(((it + i) / nst) & 1));
+                    const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)st * n);
 #pragma unroll
-                for (int w = 0; w < kFusedWarps / 4; ++w) {
-                    const float4 t4 = rb4[w];
-                    v[4 * w] = t4.x;
-                    v[4 * w + 1] = t4.y;
-                    v[4 * w + 2] = t4.z;
-                    v[4 * w + 3] = t4.w;
+                    for (int q = 0; q < QC; ++q) {
+                        const int64_t c = tid + (int64_t)kFusedThreads * q;
+                        a[i][q] = c < nv ? S4[c] : zero4();
+                    }
+                } else {
+#pragma unroll
+                    for (int q = 0; q < QC; ++q) a[i][q] = zero4();
                 }
-                const float t = pair_tree<kFusedWarps>(v);  // t_r = A_r . x
+            }
+            // partial dots of this thread's columns, CR rows at once
+            float d[CR];
 #pragma unroll
-                for (int q = 0; q < QC; ++q) fma4s(yr[q], a[i][q], t);  // y += A_r^T t_r
+            for (int i = 0; i < CR; ++i) {
+                float4 acc = zero4();
+#pragma unroll
+                for (int q = 0; q < QC; ++q) fma4(acc, a[i][q], xr[q]);
+                d[i] = hsum4(acc);
+            }
+#pragma unroll
+            for (int o = 16; o > 0; o >>= 1)
+#pragma unroll
+                for (int i = 0; i < CR; ++i) d[i] = __fadd_rn(d[i], __shfl_xor_sync(0xffffffffu, d[i], o));
+            if (lane == 0) {
+#pragma unroll
+                for (int i = 0; i < CR; ++i) rb[i * kFusedWarps + warp] = d[i];
             }
         }
+        // rank-1 updates of the previous step: y += A_r^T t_r
+        if (prow > 0) {
+            const float *pb = red + (buf ^ 1) * CR * kFusedWarps;
+#pragma unroll
+            for (int i = 0; i < CR; ++i) {
+                if (i < prow) {
+                    float v[kFusedWarps];
+                    const float4 *rb4 = reinterpret_cast<const float4 *>(pb + i * kFusedWarps);
+#pragma unroll
+                    for (int w = 0; w < kFusedWarps / 4; ++w) {
+                        const float4 t4 = rb4[w];
+                        v[4 * w] = t4.x;
+                        v[4 * w + 1] = t4.y;
+                        v[4 * w + 2] = t4.z;
+                        v[4 * w + 3] = t4.w;
+                    }
+                    const float t = pair_tree<kFusedWarps>(v);  // t_r = A_r . x
+#pragma unroll
+                    for (int q = 0; q < QC; ++q) fma4s(yr[q], ap[i][q], t);
+                }
+            }
+        }
+        if (rows == 0) break;
+#pragma unroll
+        for (int i = 0; i < CR; ++i)
+#pragma unroll
+            for (int q = 0; q < QC; ++q) ap[i][q] = a[i][q];
+        prow = rows;
+        prev_r = r;
         it += rows;
     }
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
@@ -405,11 +531,11 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     }
 
     // ---- second stage in the same launch: grid barrier, then every block sums
-    // tiles of 32 float4 columns over all G partial rows in a fixed order ----
+    // a slice of the columns over all G partial rows in a fixed order ----
     grid_barrier(gbar);
-    float *part = stage0;  // the ring is drained: reuse it for the tile partials
-    for (int64_t c0 = (int64_t)blockIdx.x * 32; c0 < nv; c0 += (int64_t)gridDim.x * 32)
-        colsum_tile<4, kFusedWarps>((int)gridDim.x, nv, P, y, c0, part);
+    // every block sums its own slice of columns (the drained ring holds the split sums)
+    const int64_t c0 = nv * blockIdx.x / gridDim.x, c1 = nv * (blockIdx.x + 1) / gridDim.x;
+    colsum_slice((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0));
     grid_depart(gbar);
 }
 
@@ -449,9 +575,9 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, y, gbar, (int)G, s);
     LIFT_FUSED_CASE(1, 4)
     LIFT_FUSED_CASE(2, 4)
-    LIFT_FUSED_CASE(4, 4)
+    LIFT_FUSED_CASE(2, 2)
     LIFT_FUSED_CASE(4, 2)
-    LIFT_FUSED_CASE(8, 2)
+    LIFT_FUSED_CASE(4, 1)
     LIFT_FUSED_CASE(8, 1)
 #undef LIFT_FUSED_CASE
     return e;

@@ -135,7 +135,14 @@ int lift_gemv_tuned(int64_t m, int64_t n, const float *A, const float *x, float 
     cfg.blocks = blocks;
     cfg.xsmem = xsmem;
     cfg.lb = lb;
-    return cuda_status(lift::launch_gemv(d, 1, m, n, A, nullptr, x, y, 1.f, 0.f, cfg, (cudaStream_t)stream));
+    lift::GemvArgs g;
+    g.m = m;
+    g.n = n;
+    g.lda = n;
+    g.A = A;
+    g.x = x;
+    g.y = y;
+    return cuda_status(lift::launch_gemv(d, g, cfg, (cudaStream_t)stream));
 }
 
 int lift_gemv(int64_t m, int64_t n, const float *A, const float *x, float *y, lift_stream_t stream) {
@@ -156,7 +163,19 @@ int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *A, float 
     cfg.blocks = blocks;
     cfg.xsmem = xsmem;
     cfg.lb = lb;
-    return cuda_status(lift::launch_gemv(d, 2, m, n, A, B, x, y, alpha, beta, cfg, (cudaStream_t)stream));
+    lift::GemvArgs g;
+    g.nmat = 2;
+    g.m = m;
+    g.n = n;
+    g.lda = n;
+    g.A = A;
+    g.B = B;
+    g.x = x;
+    g.y = y;
+    g.alpha = alpha;
+    g.beta = beta;
+    g.epi = lift::kEpiSum2;
+    return cuda_status(lift::launch_gemv(d, g, cfg, (cudaStream_t)stream));
 }
 
 int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B, const float *x,
@@ -202,6 +221,66 @@ int lift_atax_algo_run(int algo, int64_t m, int64_t n, const float *A, const flo
 int lift_atax(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
               size_t workspace_bytes, lift_stream_t stream) {
     return lift_atax_algo_run(LIFT_ATAX_AUTO, m, n, A, x, y, workspace, workspace_bytes, stream);
+}
+
+// (layout, trans) -> does the row-major kernel walk rows of the stored matrix (false)
+// or its columns (true)?  Column-major A is the row-major A^T.
+static bool sgemv_colpath(int layout, int trans) { return (layout == 0) == (trans == 1); }
+
+size_t lift_sgemv_workspace_bytes(int layout, int trans, int64_t m, int64_t n) {
+    if (!size_ok(m, n) || (layout != 0 && layout != 1) || (trans != 0 && trans != 1)) return 0;
+    if (!sgemv_colpath(layout, trans)) return 0;
+    // stored row-major matrix R = (layout 0 ? A : A^T): rows x cols; the column path reduces over rows
+    const int64_t cols = layout == 0 ? n : m;
+    const int64_t rows = layout == 0 ? m : n;
+    return lift::gemv_t_ws_bytes(rows, cols);
+}
+
+int lift_sgemv(int layout, int trans, int64_t m, int64_t n, float alpha, const float *A, int64_t lda, const float *x,
+               float beta, float *y, void *workspace, size_t workspace_bytes, lift_stream_t stream) {
+    if ((layout != 0 && layout != 1) || (trans != 0 && trans != 1)) return LIFT_ERR_BAD_SIZE;
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    // the stored matrix as row-major R: rows x cols with row stride lda
+    const int64_t rows = layout == 0 ? m : n, cols = layout == 0 ? n : m;
+    if (lda < (cols > 1 ? cols : 1)) return LIFT_ERR_BAD_SIZE;
+    if (rows > 0 && !size_ok(rows, lda)) return LIFT_ERR_BAD_SIZE;
+    const int64_t xlen = trans == 0 ? n : m, ylen = trans == 0 ? m : n;
+    if (ylen > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
+    if (m > 0 && n > 0 && (A == nullptr || x == nullptr)) return LIFT_ERR_NULL_PTR;
+    if (ylen > 0 && mis4(y)) return LIFT_ERR_MISALIGNED;
+    if (m > 0 && n > 0 && (mis4(A) || mis4(x))) return LIFT_ERR_MISALIGNED;
+    const bool colpath = sgemv_colpath(layout, trans);
+    const size_t need = lift_sgemv_workspace_bytes(layout, trans, m, n);
+    if (need > 0 && (workspace == nullptr || workspace_bytes < need || (reinterpret_cast<uintptr_t>(workspace) & 15)))
+        return LIFT_ERR_WORKSPACE;
+    if (ylen > 0) {
+        const uint64_t abytes = rows > 0 ? ((uint64_t)(rows - 1) * (uint64_t)lda + (uint64_t)cols) * 4 : 0;
+        const Range ry = rng(y, (uint64_t)ylen * 4);
+        if (overlap(ry, rng(A, abytes)) || overlap(ry, rng(x, (uint64_t)xlen * 4)) ||
+            (need > 0 && overlap(ry, rng(workspace, workspace_bytes))))
+            return LIFT_ERR_ALIAS;
+        if (need > 0 && (overlap(rng(workspace, workspace_bytes), rng(A, abytes)) ||
+                         overlap(rng(workspace, workspace_bytes), rng(x, (uint64_t)xlen * 4))))
+            return LIFT_ERR_ALIAS;
+    }
+    if (ylen == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    if (colpath)  // y (length cols) = alpha * R^T x + beta * y
+        return cuda_status(lift::launch_gemv_t(d, rows, cols, lda, alpha, A, x, beta, y, workspace,
+                                               (cudaStream_t)stream));
+    lift::GemvArgs g;  // y (length rows) = alpha * R x + beta * y
+    g.m = rows;
+    g.n = cols;
+    g.lda = lda;
+    g.A = A;
+    g.x = x;
+    g.y = y;
+    g.alpha = alpha;
+    g.beta = beta;
+    g.epi = lift::kEpiAxpby;
+    return cuda_status(lift::launch_gemv(d, g, lift::GemvConfig{}, (cudaStream_t)stream));
 }
 
 int lift_partial_dot(int64_t n, const float *x, const float *y, float *z, int contract, lift_stream_t stream) {

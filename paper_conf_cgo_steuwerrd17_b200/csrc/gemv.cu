@@ -63,9 +63,10 @@ __host__ __device__ constexpr int gemv_x_offset() {
 }
 
 template <int NMAT, int VEC, int WPR, int RG, bool XSMEM, int LB>
-__global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, const float *__restrict__ A,
-                                                        const float *__restrict__ B, const float *__restrict__ x,
-                                                        float *__restrict__ y, float alpha, float beta) {
+__global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, int64_t lda,
+                                                        const float *__restrict__ A, const float *__restrict__ B,
+                                                        const float *__restrict__ x, float *__restrict__ y,
+                                                        float alpha, float beta, int epi) {
     using V = Vec<VEC>;
     using T = typename V::T;
     constexpr int KQ = kSlices / WPR;                                 // slices per warp
@@ -98,8 +99,8 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
     // so a warp keeps loads in flight while it reduces a finished row.
     // Full batches use compile-time offsets and no predicates.
     auto load_batch = [&](int64_t r, int64_t k0, T (&dst)[NMAT][UK][KQ]) {
-        const T *Ar = reinterpret_cast<const T *>(A + r * n) + (kVLanes * k0 + lane_off);
-        const T *Br = (NMAT == 2) ? reinterpret_cast<const T *>(B + r * n) + (kVLanes * k0 + lane_off) : nullptr;
+        const T *Ar = reinterpret_cast<const T *>(A + r * lda) + (kVLanes * k0 + lane_off);
+        const T *Br = (NMAT == 2) ? reinterpret_cast<const T *>(B + r * lda) + (kVLanes * k0 + lane_off) : nullptr;
         if (k0 + UK <= kfull) {
 #pragma unroll
             for (int u = 0; u < UK; ++u)
@@ -211,10 +212,15 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
                     buf ^= 1;
                 }
                 if (writer) {
-                    if constexpr (NMAT == 1)
-                        y[row] = s[0];
-                    else
+                    if constexpr (NMAT == 1) {
+                        if (epi == kEpiStore)
+                            y[row] = s[0];
+                        else  // kEpiAxpby (BLAS: y is not read when beta == 0)
+                            y[row] = beta == 0.f ? __fmul_rn(alpha, s[0])
+                                                 : __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, y[row]));
+                    } else {
                         y[row] = __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, s[1]));
+                    }
                 }
                 if (nrow >= m) break;
             }
@@ -239,11 +245,10 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, c
 // ---------------------------------------------------------------------------
 
 template <int NMAT, int VEC, int WPR, int RG, bool XSMEM, int LB>
-static cudaError_t run_gemv(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *B,
-                            const float *x, float *y, float alpha, float beta, int blocks, cudaStream_t s) {
+static cudaError_t run_gemv(const DeviceInfo &d, const GemvArgs &a, int blocks, cudaStream_t s) {
     auto kern = k_gemv<NMAT, VEC, WPR, RG, XSMEM, LB>;
     constexpr int threads = RG * WPR * kWarp;
-    size_t smem = gemv_x_offset<NMAT, RG>() + (XSMEM ? (size_t)n * 4 : 0);
+    size_t smem = gemv_x_offset<NMAT, RG>() + (XSMEM ? (size_t)a.n * 4 : 0);
     if (smem > 48 * 1024) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         if (e != cudaSuccess) return e;
@@ -252,23 +257,22 @@ static cudaError_t run_gemv(const DeviceInfo &d, int64_t m, int64_t n, const flo
     cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, threads, smem);
     if (e != cudaSuccess) return e;
     if (per_sm < 1) return cudaErrorInvalidConfiguration;
-    const int64_t groups = (m + RG - 1) / RG;
+    const int64_t groups = (a.m + RG - 1) / RG;
     int64_t cap = (int64_t)per_sm * d.sms;
     int64_t g = blocks > 0 ? blocks : (groups < cap ? groups : cap);
     if (g < 1) g = 1;
-    kern<<<(unsigned)g, threads, smem, s>>>(m, n, A, B, x, y, alpha, beta);
+    kern<<<(unsigned)g, threads, smem, s>>>(a.m, a.n, a.lda, a.A, a.B, a.x, a.y, a.alpha, a.beta, a.epi);
     return cudaGetLastError();
 }
 
 template <int NMAT, int VEC, bool XSMEM>
-static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int lb, int64_t m, int64_t n, const float *A,
-                                const float *B, const float *x, float *y, float alpha, float beta, int blocks,
+static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int lb, const GemvArgs &a, int blocks,
                                 cudaStream_t s) {
     // block = RG row groups of WPR warps; 256..1024 threads
-#define LIFT_GEMV_CASE(W, R)                                                                           \
-    if (wpr == W && rg == R) {                                                                         \
-        if (lb == 8) return run_gemv<NMAT, VEC, W, R, XSMEM, 8>(d, m, n, A, B, x, y, alpha, beta, blocks, s); \
-        return run_gemv<NMAT, VEC, W, R, XSMEM, 4>(d, m, n, A, B, x, y, alpha, beta, blocks, s);            \
+#define LIFT_GEMV_CASE(W, R)                                                         \
+    if (wpr == W && rg == R) {                                                       \
+        if (lb == 8) return run_gemv<NMAT, VEC, W, R, XSMEM, 8>(d, a, blocks, s);    \
+        return run_gemv<NMAT, VEC, W, R, XSMEM, 4>(d, a, blocks, s);                 \
     }
     LIFT_GEMV_CASE(8, 1)
     LIFT_GEMV_CASE(8, 2)
@@ -281,14 +285,16 @@ static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int lb, in
     return cudaErrorInvalidValue;
 }
 
-cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, const float *A, const float *B,
-                        const float *x, float *y, float alpha, float beta, GemvConfig cfg, cudaStream_t s) {
+cudaError_t launch_gemv(const DeviceInfo &d, const GemvArgs &a, GemvConfig cfg, cudaStream_t s) {
+    const int64_t m = a.m, n = a.n;
     if (m == 0) return cudaSuccess;
-    if (n == 0) return cudaMemsetAsync(y, 0, (size_t)m * sizeof(float), s);
-    uintptr_t orr = reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
-                    (nmat == 2 ? reinterpret_cast<uintptr_t>(B) : 0);
-    const bool vec = (n % 4 == 0) && (orr & 15) == 0;
-    // x in smem when it fits next to the red buffers (bulk copy needs 16-B units)
+    if (n == 0) {
+        if (a.epi == kEpiStore) return cudaMemsetAsync(a.y, 0, (size_t)m * sizeof(float), s);
+        // y = 0 + beta*y (and 0 when beta == 0): handled by the kernel with an empty row
+    }
+    uintptr_t orr = reinterpret_cast<uintptr_t>(a.A) | reinterpret_cast<uintptr_t>(a.x) |
+                    (a.nmat == 2 ? reinterpret_cast<uintptr_t>(a.B) : 0);
+    const bool vec = n > 0 && (n % 4 == 0) && (a.lda % 4 == 0) && (orr & 15) == 0;
     const size_t x_bytes = (size_t)n * 4;
     // Defaults from the B200 sweep (tools/sweep.py, profiles/r01b_sweep.txt): one row per
     // 256-thread block (8 warps x 1 slice each), 4 vector loads per lane per batch, x in
@@ -311,16 +317,16 @@ cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, con
     if (lb == 0) lb = 4;
     if (lb != 4 && lb != 8) return cudaErrorInvalidValue;
     if (vec) {
-        if (nmat == 1)
-            return xsmem ? dispatch_wpr<1, 4, true>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
-                         : dispatch_wpr<1, 4, false>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
-        return xsmem ? dispatch_wpr<2, 4, true>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s)
-                     : dispatch_wpr<2, 4, false>(d, wpr, rg, lb, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+        if (a.nmat == 1)
+            return xsmem ? dispatch_wpr<1, 4, true>(d, wpr, rg, lb, a, cfg.blocks, s)
+                         : dispatch_wpr<1, 4, false>(d, wpr, rg, lb, a, cfg.blocks, s);
+        return xsmem ? dispatch_wpr<2, 4, true>(d, wpr, rg, lb, a, cfg.blocks, s)
+                     : dispatch_wpr<2, 4, false>(d, wpr, rg, lb, a, cfg.blocks, s);
     }
-    // scalar path (n % 4 != 0 or misaligned): one shape
+    // scalar path (n % 4 != 0, lda % 4 != 0 or misaligned): one shape
     if (wpr != 1 || rg != 8 || lb != 4) return cudaErrorInvalidValue;
-    if (nmat == 1) return run_gemv<1, 1, 1, 8, false, 4>(d, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
-    return run_gemv<2, 1, 1, 8, false, 4>(d, m, n, A, B, x, y, alpha, beta, cfg.blocks, s);
+    if (a.nmat == 1) return run_gemv<1, 1, 1, 8, false, 4>(d, a, cfg.blocks, s);
+    return run_gemv<2, 1, 1, 8, false, 4>(d, a, cfg.blocks, s);
 }
 
 }  // namespace lift

@@ -34,9 +34,22 @@ struct GemvConfig {
     int xsmem = -1;  // 1 = stage x in smem by bulk copy, 0 = read x through L1, -1 = auto
     int lb = 0;      // vector loads per lane per batch (4 or 8; x2 in flight with the prefetch); 0 = auto
 };
-// nmat = 1: y = A x;  nmat = 2: y = alpha A x + beta B x
-cudaError_t launch_gemv(const DeviceInfo &d, int nmat, int64_t m, int64_t n, const float *A, const float *B,
-                        const float *x, float *y, float alpha, float beta, GemvConfig cfg, cudaStream_t s);
+// Epilogue applied to the row sums (sA, sB):
+//   kEpiStore   y_i = sA                                  (GEMV)
+//   kEpiAxpby   y_i = alpha*sA + beta*y_i  (y not read when beta == 0; BLAS SGEMV)
+//   kEpiSum2    y_i = alpha*sA + beta*sB                  (GESUMMV, nmat = 2)
+// Each product is rounded, then one rounded add.
+enum GemvEpi { kEpiStore = 0, kEpiAxpby = 1, kEpiSum2 = 2 };
+struct GemvArgs {
+    int nmat = 1;            // 1: A only; 2: A and B (zipped rows)
+    int64_t m = 0, n = 0;    // rows, columns
+    int64_t lda = 0;         // row stride of A and B in floats (>= n)
+    const float *A = nullptr, *B = nullptr, *x = nullptr;
+    float *y = nullptr;
+    float alpha = 1.f, beta = 0.f;
+    int epi = kEpiStore;
+};
+cudaError_t launch_gemv(const DeviceInfo &d, const GemvArgs &a, GemvConfig cfg, cudaStream_t s);
 
 // ---- ATAX ----------------------------------------------------------------------
 size_t atax_twopass_ws_bytes(int64_t m, int64_t n);
@@ -45,6 +58,11 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16);
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16);
 cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
                                 float *y, void *ws, cudaStream_t s);
+// y = alpha * A^T x + beta * y  (A m x n row-major with stride lda; x in R^m, y in R^n):
+// column-blocked partials over row splits + fixed-order column sum with the epilogue
+size_t gemv_t_ws_bytes(int64_t m, int64_t n);
+cudaError_t launch_gemv_t(const DeviceInfo &d, int64_t m, int64_t n, int64_t lda, float alpha, const float *A,
+                          const float *x, float beta, float *y, void *ws, cudaStream_t s);
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
                               float *y, void *ws, cudaStream_t s);
 

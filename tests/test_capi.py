@@ -173,3 +173,17 @@ def test_listing1_validation():
     assert L.lift_dot_listing1(1000, X_, Y_, P * 300, W_, ws - 1, 1, None) == WS
     assert L.lift_dot_listing1(1000, X_, Y_, W_ + 8, W_, ws, 1, None) == ALIAS
     assert L.lift_dot_listing1(1000, X_, Y_, None, W_, ws, 1, None) == NULL
+
+
+def test_sgemv_validation():
+    assert L.lift_sgemv_workspace_bytes(0, 0, 100, 50) == 0          # row-major, no transpose: no workspace
+    assert L.lift_sgemv_workspace_bytes(0, 1, 100, 50) > 0
+    assert L.lift_sgemv_workspace_bytes(1, 0, 100, 50) > 0           # column-major = transposed rows
+    assert L.lift_sgemv_workspace_bytes(1, 1, 100, 50) == 0
+    assert L.lift_sgemv(2, 0, 4, 4, 1.0, A_, 4, X_, 0.0, Y_, None, 0, None) == SIZE
+    assert L.lift_sgemv(0, 0, 4, 4, 1.0, A_, 3, X_, 0.0, Y_, None, 0, None) == SIZE   # lda < n
+    assert L.lift_sgemv(1, 1, 4, 6, 1.0, A_, 3, X_, 0.0, Y_, None, 0, None) == SIZE   # col-major lda < m
+    assert L.lift_sgemv(0, 0, 4, 4, 1.0, None, 4, X_, 0.0, Y_, None, 0, None) == NULL
+    assert L.lift_sgemv(0, 1, 4, 4, 1.0, A_, 4, X_, 0.0, Y_, None, 0, None) == WS
+    assert L.lift_sgemv(0, 0, 4, 4, 1.0, A_, 8, X_, 0.0, A_ + 4 * 9, None, 0, None) == ALIAS
+    assert L.lift_sgemv(0, 0, 0, 4, 1.0, None, 4, None, 0.0, None, None, 0, None) == OK

@@ -439,3 +439,49 @@ def test_dot_listing1_close_to_fp64_and_empty():
     s64, mag = oracle.dot(x, y)
     # depth: 2 pair folds + 6 tree levels per stage, 3 stages at 2^20
     assert abs(oracle.dot_listing1_f32(x, y) - s64) <= 24 * 2.0 ** -24 * mag
+
+
+# ---------------------------------------------------------------------------
+# BLAS SGEMV (NEXT-4; CLBlast contract for Table 1's GEMV)
+# ---------------------------------------------------------------------------
+
+def _stored(Amat, layout, lda):
+    """Store the logical m x n matrix in a padded buffer (padding = NaN, never read)."""
+    m, n = Amat.shape
+    if layout == 0:
+        buf = np.full((m, lda), np.nan, np.float32)
+        buf[:, :n] = Amat
+    else:
+        buf = np.full((n, lda), np.nan, np.float32)
+        buf[:, :m] = Amat.T
+    return buf
+
+
+@pytest.mark.parametrize("layout", [0, 1])
+@pytest.mark.parametrize("trans", [0, 1])
+@pytest.mark.parametrize("alpha,beta", [(1.0, 0.0), (-0.5, 2.0), (1.5, 1.2)])
+def test_sgemv_bruteforce_fraction(layout, trans, alpha, beta):
+    m, n = 5, 7
+    Am = rand_f32(2, (m, n))
+    lda = (n if layout == 0 else m) + 3
+    buf = _stored(Am, layout, lda)
+    x = rand_f32(0, (m if trans else n,))
+    yin = rand_f32(9, (n if trans else m,))
+    y, mag = oracle.sgemv(layout, trans, m, n, alpha, buf, lda, x, beta, yin)
+    opA = Am.T if trans else Am
+    a32, b32 = F(np.float32(alpha)), F(np.float32(beta))
+    exact = [a32 * s + (b32 * F(yv) if beta != 0 else 0) for s, yv in zip(exact_matvec(opA, x), yin)]
+    assert np.all(np.isfinite(y))  # the NaN padding is never read
+    assert_close_exact(y, exact, opA.shape[1] + 2, mag)
+
+
+def test_sgemv_reduces_to_gemv_and_ignores_y_when_beta_zero():
+    m, n = 6, 9
+    Am = rand_f32(2, (m, n))
+    x = rand_f32(0, (n,))
+    y, _ = oracle.sgemv(0, 0, m, n, 1.0, Am, n, x, 0.0, np.full(m, np.nan, np.float32))
+    g, _ = oracle.gemv(Am, x)
+    assert np.array_equal(y, g)
+    # column-major storage of A^T read as row-major A: same result
+    yt, _ = oracle.sgemv(1, 1, n, m, 1.0, Am, n, x, 0.0)
+    assert np.array_equal(yt, g)

@@ -400,3 +400,37 @@ def test_partial_dot_unaligned(cuda_device):
     got = lift.lift_partial_dot(x, y).cpu().numpy()
     ref = oracle.partial_dot_listing1_f32(x.cpu().numpy(), y.cpu().numpy())
     assert np.array_equal(got.view(np.uint32), ref.view(np.uint32))
+
+
+# ===================================================================== BLAS SGEMV (NEXT-4)
+@pytest.mark.parametrize("layout", ["row", "col"])
+@pytest.mark.parametrize("trans", [False, True])
+@pytest.mark.parametrize("m,n,pad", [(300, 1000, 0), (333, 517, 3), (4096, 4096, 4), (7, 3, 1), (0, 5, 0), (5, 0, 0)])
+@pytest.mark.parametrize("alpha,beta", [(1.0, 0.0), (1.5, 1.2), (-2.0, 0.5)])
+def test_sgemv_parity(cuda_device, layout, trans, m, n, pad, alpha, beta):
+    lay = 0 if layout == "row" else 1
+    rows, cols = (m, n) if lay == 0 else (n, m)
+    lda = max(cols, 1) + pad
+    buf = synth.numpy_uniform(synth.SEED_A, 0, rows * lda).reshape(rows, lda) if rows else np.zeros((0, lda), np.float32)
+    x = rand(synth.SEED_X, (m if trans else n,))
+    ylen = n if trans else m
+    yin = rand(9, (ylen,))
+    yd = dev_np(yin, cuda_device)
+    if beta == 0.0:
+        yd.fill_(float("nan"))  # must not be read
+    lift.lift_sgemv(alpha, dev_np(buf, cuda_device), dev_np(x, cuda_device), beta, yd, trans=trans, layout=layout,
+                    lda=lda, shape=(m, n))
+    ref, mag = oracle.sgemv(lay, int(trans), m, n, alpha, buf, lda, x, beta, yin)
+    assert_tol(yd.cpu().numpy(), ref, mag, f"sgemv {layout} trans={trans} {m}x{n}")
+
+
+def test_sgemv_alpha1_beta0_is_gemv_bitwise(cuda_device):
+    m, n = 777, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    assert torch.equal(lift.lift_sgemv(1.0, A, x), lift.lift_gemv(A, x))
+    # y = 2*(Ax) - 1*y applied twice from y = Ax gives Ax exactly (power-of-two scalings)
+    y = lift.lift_gemv(A, x)
+    ref = y.clone()
+    lift.lift_sgemv(2.0, A, x, -1.0, y)
+    assert torch.equal(y, ref)
