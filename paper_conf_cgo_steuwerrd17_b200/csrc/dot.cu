@@ -114,21 +114,24 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
 
 cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
                        void *workspace, cudaStream_t s) {
-    constexpr int TPB = 512;
+    // B200 read sweep (tools/readbw.cu, profiles/r01j_readbw.txt): 256-thread blocks with
+    // U = 4 float4 pairs in flight per thread and TWO waves of blocks stream fastest
+    // (7.48 TB/s vs 7.39 for 512 threads / one wave); later blocks fill the tail.
+    constexpr int TPB = 256;
     constexpr int U = 4;
+    constexpr int kWaves = 2;
     unsigned int *ticket = static_cast<unsigned int *>(workspace);
     float *partials = reinterpret_cast<float *>(static_cast<char *>(workspace) + kDotTicketBytes);
     const bool vec = ((reinterpret_cast<uintptr_t>(x) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
     const int64_t units = vec ? (n >> 2) : n;
-    // enough blocks to give every thread >= 1 unit; at most ONE resident wave
-    // (a second partial wave would serialise half the stream)
+    // enough blocks to give every thread >= 1 unit; at most kWaves resident waves
     int per_sm = 0;
     cudaError_t e = vec ? cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dot<TPB, U, true>, TPB, 0)
                         : cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dot<TPB, U, false>, TPB, 0);
     if (e != cudaSuccess) return e;
     if (per_sm < 1) per_sm = 1;
     int64_t want = (units + TPB - 1) / TPB;
-    int64_t cap = (int64_t)d.sms * per_sm;
+    int64_t cap = (int64_t)d.sms * per_sm * kWaves;
     if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;
     int blocks = (int)(want < 1 ? 1 : (want > cap ? cap : want));
     if (vec)

@@ -1,0 +1,135 @@
+// readbw.cu — standalone B200 read-bandwidth microbenchmark (tuning aid, not
+// part of the library): which load flavour / occupancy streams HBM fastest?
+// Each variant sums two 4 GiB fp32 arrays (x.y) and is timed with CUDA events
+// (best of 5 after 2 warm-ups).  Build: nvcc -gencode arch=compute_100a,code=sm_100a -O3
+#include <cstdio>
+#include <cstdint>
+#include <cuda_runtime.h>
+
+__device__ __forceinline__ float4 ld4_na(const float4 *p) {
+    float4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.f32 {%0,%1,%2,%3}, [%4];"
+                 : "=f"(r.x), "=f"(r.y), "=f"(r.z), "=f"(r.w) : "l"(p));
+    return r;
+}
+__device__ __forceinline__ float4 ld4_pf(const float4 *p) {
+    float4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.L2::256B.v4.f32 {%0,%1,%2,%3}, [%4];"
+                 : "=f"(r.x), "=f"(r.y), "=f"(r.z), "=f"(r.w) : "l"(p));
+    return r;
+}
+struct f8 { float v[8]; };
+__device__ __forceinline__ f8 ld8(const float *p) {
+    f8 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v8.f32 {%0,%1,%2,%3,%4,%5,%6,%7}, [%8];"
+                 : "=f"(r.v[0]), "=f"(r.v[1]), "=f"(r.v[2]), "=f"(r.v[3]), "=f"(r.v[4]), "=f"(r.v[5]),
+                   "=f"(r.v[6]), "=f"(r.v[7]) : "l"(p));
+    return r;
+}
+__device__ __forceinline__ f8 ld8_ef(const float *p) {
+    f8 r;
+    asm volatile("ld.global.nc.L1::no_allocate.L2::evict_first.v8.f32 {%0,%1,%2,%3,%4,%5,%6,%7}, [%8];"
+                 : "=f"(r.v[0]), "=f"(r.v[1]), "=f"(r.v[2]), "=f"(r.v[3]), "=f"(r.v[4]), "=f"(r.v[5]),
+                   "=f"(r.v[6]), "=f"(r.v[7]) : "l"(p));
+    return r;
+}
+
+template <int U, int MODE>
+__global__ void k4(int64_t n4, const float4 *x, const float4 *y, float *out) {
+    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+    int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    float4 acc[U];
+    for (int u = 0; u < U; ++u) acc[u] = make_float4(0, 0, 0, 0);
+    for (; i + (U - 1) * stride < n4; i += U * stride) {
+        float4 a[U], b[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            a[u] = MODE == 0 ? ld4_na(x + i + u * stride) : ld4_pf(x + i + u * stride);
+            b[u] = MODE == 0 ? ld4_na(y + i + u * stride) : ld4_pf(y + i + u * stride);
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            acc[u].x = fmaf(a[u].x, b[u].x, acc[u].x);
+            acc[u].y = fmaf(a[u].y, b[u].y, acc[u].y);
+            acc[u].z = fmaf(a[u].z, b[u].z, acc[u].z);
+            acc[u].w = fmaf(a[u].w, b[u].w, acc[u].w);
+        }
+    }
+    float s = 0;
+    for (int u = 0; u < U; ++u) s += acc[u].x + acc[u].y + acc[u].z + acc[u].w;
+    if (s == 12345.f) out[0] = s;  // keep the loads alive
+}
+
+template <int U, int MODE>
+__global__ void k8(int64_t n8, const float *x, const float *y, float *out) {
+    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+    int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    float acc[8] = {0, 0, 0, 0, 0, 0, 0, 0};
+    for (; i + (U - 1) * stride < n8; i += U * stride) {
+        f8 a[U], b[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            a[u] = MODE == 0 ? ld8(x + 8 * (i + u * stride)) : ld8_ef(x + 8 * (i + u * stride));
+            b[u] = MODE == 0 ? ld8(y + 8 * (i + u * stride)) : ld8_ef(y + 8 * (i + u * stride));
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u)
+#pragma unroll
+            for (int k = 0; k < 8; ++k) acc[k] = fmaf(a[u].v[k], b[u].v[k], acc[k]);
+    }
+    float s = 0;
+    for (int k = 0; k < 8; ++k) s += acc[k];
+    if (s == 12345.f) out[0] = s;
+}
+
+template <typename K, typename... Args>
+static void run(const char *name, K kern, int tpb, int64_t bytes, Args... args) {
+    int per_sm = 0;
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, tpb, 0);
+    int sms = 0;
+    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
+    for (int mult : {1, 2}) {
+        int grid = per_sm * sms * mult;
+        cudaEvent_t a, b;
+        cudaEventCreate(&a);
+        cudaEventCreate(&b);
+        float best = 1e30f;
+        for (int it = 0; it < 7; ++it) {
+            cudaEventRecord(a);
+            kern<<<grid, tpb>>>(args...);
+            cudaEventRecord(b);
+            cudaEventSynchronize(b);
+            float ms;
+            cudaEventElapsedTime(&ms, a, b);
+            if (it >= 2 && ms < best) best = ms;
+        }
+        printf("%-34s tpb %4d  per_sm %2d  grid x%d  %9.1f us  %7.1f GB/s\n", name, tpb, per_sm, mult, best * 1e3,
+               bytes / (best * 1e-3) / 1e9);
+    }
+}
+
+int main() {
+    const int64_t n = (int64_t)1 << 30;  // 4 GiB per array
+    float *x, *y, *out;
+    cudaMalloc(&x, n * 4);
+    cudaMalloc(&y, n * 4);
+    cudaMalloc(&out, 64);
+    cudaMemset(x, 0, n * 4);
+    cudaMemset(y, 0, n * 4);
+    const int64_t bytes = 8 * n;
+    const float4 *x4 = (const float4 *)x, *y4 = (const float4 *)y;
+    run("v4 na U4", k4<4, 0>, 512, bytes, n / 4, x4, y4, out);
+    run("v4 na U4", k4<4, 0>, 256, bytes, n / 4, x4, y4, out);
+    run("v4 na U8", k4<8, 0>, 256, bytes, n / 4, x4, y4, out);
+    run("v4 na U2", k4<2, 0>, 512, bytes, n / 4, x4, y4, out);
+    run("v4 L2::256B U4", k4<4, 1>, 512, bytes, n / 4, x4, y4, out);
+    run("v4 L2::256B U8", k4<8, 1>, 256, bytes, n / 4, x4, y4, out);
+    run("v8 na U2", k8<2, 0>, 512, bytes, n / 8, x, y, out);
+    run("v8 na U4", k8<4, 0>, 256, bytes, n / 8, x, y, out);
+    run("v8 na U4", k8<4, 0>, 512, bytes, n / 8, x, y, out);
+    run("v8 evict_first U4", k8<4, 1>, 256, bytes, n / 8, x, y, out);
+    run("v8 evict_first U2", k8<2, 1>, 512, bytes, n / 8, x, y, out);
+    cudaError_t e = cudaGetLastError();
+    printf("status %s\n", cudaGetErrorString(e));
+    return 0;
+}

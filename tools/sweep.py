@@ -39,6 +39,7 @@ def graph_time(calls, reps=3):
 
 
 CONFIGS = [(8, 1), (8, 2), (4, 2), (4, 4), (2, 4), (2, 8), (1, 8)]
+FULL = "--full" in sys.argv
 
 
 def sweep(op, m, n, nsets, ncalls=24):
@@ -61,7 +62,7 @@ def sweep(op, m, n, nsets, ncalls=24):
                                           lift.lift_gesummv(1.5, A, 1.2, B, x, out=y)))
                        for A, B in (sets * ncalls)[:ncalls]])
     print(f"{op} {m}x{n} auto: {auto:8.2f} us  {nbytes / auto / 1e3:7.1f} GB/s", flush=True)
-    for (wpr, rg), xs, lb in itertools.product(CONFIGS, (0, 1), (4, 8)):
+    for (wpr, rg), xs, lb in (itertools.product(CONFIGS, (0, 1), (4, 8)) if FULL else ()):
         try:
             calls = [mk(A, B, wpr=wpr, rg=rg, xsmem=xs, lb=lb) for A, B in (sets * ncalls)[:ncalls]]
             t = graph_time(calls)
@@ -70,6 +71,12 @@ def sweep(op, m, n, nsets, ncalls=24):
             continue
         res.append((t, wpr, rg, xs, lb))
         print(f"  wpr={wpr} rg={rg} xs={xs} lb={lb}: {t:8.2f} us  {nbytes / t / 1e3:7.1f} GB/s", flush=True)
+    for blocks in (296, 444, 592, 888, 1184, 1776, 2368):
+        for xs in (0, 1):
+            calls = [mk(A, B, wpr=8, rg=1, xsmem=xs, lb=4, blocks=blocks) for A, B in (sets * ncalls)[:ncalls]]
+            t = graph_time(calls)
+            res.append((t, 8, 1, xs, 4, blocks))
+            print(f"  wpr=8 rg=1 xs={xs} lb=4 blocks={blocks}: {t:8.2f} us  {nbytes / t / 1e3:7.1f} GB/s", flush=True)
     res.sort()
     print(f"BEST {op} {m}x{n}: {res[0]}", flush=True)
     del sets
@@ -77,7 +84,7 @@ def sweep(op, m, n, nsets, ncalls=24):
 
 
 if __name__ == "__main__":
-    which = sys.argv[1:] or ["gemv4096", "gemv8192", "gesummv8192", "gemv65536"]
+    which = [a for a in sys.argv[1:] if not a.startswith("--")] or ["gemv4096", "gemv8192", "gesummv8192", "gemv65536"]
     if "gemv4096" in which:
         sweep("gemv", 4096, 4096, nsets=6)
     if "gemv8192" in which:
