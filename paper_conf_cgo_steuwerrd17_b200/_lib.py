@@ -29,6 +29,7 @@ LIFT_ATAX_FUSED = 1
 LIFT_ATAX_TWOPASS = 2
 
 i64 = ctypes.c_int64
+u64 = ctypes.c_uint64
 vp = ctypes.c_void_p
 f32 = ctypes.c_float
 i32 = ctypes.c_int
@@ -48,6 +49,11 @@ SIGNATURES = {
     "lift_partial_dot": (i32, [i64, vp, vp, vp, i32, vp]),
     "lift_dot_listing1_workspace_bytes": (sz, [i64]),
     "lift_dot_listing1": (i32, [i64, vp, vp, vp, vp, sz, i32, vp]),
+    "lift_exchange_bytes": (sz, [i32, i64, i32]),
+    "lift_dot_allreduce": (i32, [i64, vp, vp, vp, vp, sz, vp, i32, i32, u64, vp]),
+    "lift_gemv_allgather": (i32, [i64, i64, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, u64, vp]),
+    "lift_gesummv_allgather": (i32, [i64, i64, f32, vp, f32, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, u64, vp]),
+    "lift_atax_reduce": (i32, [i64, i64, vp, vp, vp, vp, sz, vp, i32, i32, i32, u64, i32, vp]),
     "lift_strerror": (ctypes.c_char_p, [i32]),
     "lift_last_cuda_error": (ctypes.c_char_p, []),
     "lift_version": (i32, []),

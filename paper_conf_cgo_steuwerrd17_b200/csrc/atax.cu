@@ -28,6 +28,7 @@
 #include <type_traits>
 
 #include "common.cuh"
+#include "exchange.cuh"
 #include "launch.h"
 
 namespace lift {
@@ -397,7 +398,8 @@ __device__ __forceinline__ void grid_depart(unsigned int *gbar) {
 template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
     k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
-                 float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar) {
+                 float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar, Exch ex,
+                 int dst) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
@@ -536,12 +538,53 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     // every block sums its own slice of columns (the drained ring holds the split sums)
     const int64_t c0 = nv * blockIdx.x / gridDim.x, c1 = nv * (blockIdx.x + 1) / gridDim.x;
     colsum_slice((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0));
-    grid_depart(gbar);
+    if (ex.world == 0) {
+        grid_depart(gbar);
+        return;
+    }
+    // ---- fused reduce / all-reduce over ranks (NEXT-2): push this rank's slice of
+    // A_r^T (A_r x) into row `rank` of the destination(s)' exchange area; the last
+    // block of the rank publishes; every destination block then sums its slice over
+    // the ranks in rank order (identical bits on every destination) ----
+    const float4 *y4 = reinterpret_cast<const float4 *>(y);
+    for (int q = 0; q < ex.world; ++q) {
+        if (dst >= 0 && q != dst) continue;
+        float4 *d4 = reinterpret_cast<float4 *>(exch_data(ex.peers[q], ex) + (int64_t)ex.rank * n);
+        for (int64_t c = c0 + threadIdx.x; c < c1; c += blockDim.x) d4[c] = y4[c];
+    }
+    __syncthreads();
+    __shared__ int last_block;
+    if (threadIdx.x == 0) {
+        __threadfence_system();
+        const unsigned int dep = atomicAdd(gbar + 1, 1u) + 1u;
+        last_block = dep == gridDim.x;
+        if (last_block) {  // every block has pushed (and passed the grid barrier): re-arm, publish
+            gbar[0] = 0u;
+            gbar[1] = 0u;
+            exch_signal(ex, dst);
+        }
+    }
+    if (dst >= 0 && ex.rank != dst) return;
+    if (threadIdx.x == 0) exch_wait_all(ex);
+    __syncthreads();
+    const float *src = exch_data(ex.peers[ex.rank], ex);
+    for (int64_t c = c0 + threadIdx.x; c < c1; c += blockDim.x) {
+        float4 acc = zero4();
+        for (int r = 0; r < ex.world; ++r) {
+            const float *p = src + (int64_t)r * n + 4 * c;
+            acc.x = __fadd_rn(acc.x, ld_volatile(p));
+            acc.y = __fadd_rn(acc.y, ld_volatile(p + 1));
+            acc.z = __fadd_rn(acc.z, ld_volatile(p + 2));
+            acc.w = __fadd_rn(acc.w, ld_volatile(p + 3));
+        }
+        reinterpret_cast<float4 *>(y)[c] = acc;
+    }
 }
 
 template <int QC, int CR>
 static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const float *A, const float *x, float *P,
-                             float *y, unsigned int *gbar, int blocks, cudaStream_t s) {
+                             float *y, unsigned int *gbar, int blocks, cudaStream_t s, const Exch &ex, int dst,
+                             bool cooperative) {
     auto k = k_atax_fused<QC, CR>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e != cudaSuccess) return e;
@@ -555,14 +598,14 @@ static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const flo
     attr[0].id = cudaLaunchAttributeCooperative;
     attr[0].val.cooperative = 1;
     cfg.attrs = attr;
-    cfg.numAttrs = 1;
-    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar);
+    cfg.numAttrs = cooperative ? 1 : 0;
+    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst);
 }
 
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
-                              void *ws, cudaStream_t s) {
+                              void *ws, cudaStream_t s, Exch ex, int dst, int blocks) {
     if (n == 0) return cudaSuccess;
-    if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
+    if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
     FusedPlan p;
     if (!fused_plan(n, &p)) return cudaErrorInvalidValue;
     unsigned int *gbar = static_cast<unsigned int *>(ws);
@@ -570,9 +613,14 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     int64_t G = d.sms;
     if (G > kMaxSplits) G = kMaxSplits;
     if (G > m) G = m;
+    if (G < 1) G = 1;  // m == 0 with an exchange: one block contributes a zero partial
+    // cooperative launch guarantees the co-residency the grid barrier needs; an explicit
+    // block count (tests running several ranks on one GPU) launches plainly
+    const bool cooperative = blocks <= 0;
+    if (blocks > 0) G = blocks < G ? blocks : G;
     cudaError_t e = cudaErrorInvalidValue;
 #define LIFT_FUSED_CASE(QC, CR) \
-    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, y, gbar, (int)G, s);
+    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, y, gbar, (int)G, s, ex, dst, cooperative);
     LIFT_FUSED_CASE(1, 4)
     LIFT_FUSED_CASE(2, 4)
     LIFT_FUSED_CASE(2, 2)

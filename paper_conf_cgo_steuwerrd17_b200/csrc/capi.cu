@@ -9,6 +9,7 @@
 
 #include "../../include/lift.h"
 #include "../../include/lift_tuning.h"
+#include "../../include/lift_nvlink.h"
 #include "launch.h"
 
 namespace lift {
@@ -322,6 +323,147 @@ int lift_dot_listing1(int64_t n, const float *x, const float *y, float *result, 
     if (e != cudaSuccess) return cuda_status(e);
     return cuda_status(
         lift::launch_dot_listing1(d, n, x, y, result, workspace, contract == 1, (cudaStream_t)stream));
+}
+
+// ---------------------------------------------------------------------------
+// collectives fused into the kernels (NEXT-2)
+// ---------------------------------------------------------------------------
+static int64_t exch_cap(int kind, int64_t len, int world) {
+    if (kind == LIFT_EXCH_DOT) return lift::kMaxWorld;
+    if (kind == LIFT_EXCH_GATHER) return len;
+    return (int64_t)world * len;
+}
+
+size_t lift_exchange_bytes(int kind, int64_t len, int world) {
+    if (kind < LIFT_EXCH_DOT || kind > LIFT_EXCH_REDUCE || world < 1 || world > lift::kMaxWorld || len < 0)
+        return 0;
+    if (!size_ok(exch_cap(kind, len, world), 2)) return 0;
+    const size_t b = lift::kExchHeader + 2 * (size_t)exch_cap(kind, len, world) * sizeof(float);
+    return (b + 255) / 256 * 256;
+}
+
+static int check_group(void *const *peers, int rank, int world, uint64_t epoch) {
+    if (world < 1 || world > lift::kMaxWorld || rank < 0 || rank >= world || epoch == 0) return LIFT_ERR_BAD_SIZE;
+    if (peers == nullptr) return LIFT_ERR_NULL_PTR;
+    if ((reinterpret_cast<uintptr_t>(peers) & 7) != 0) return LIFT_ERR_MISALIGNED;
+    return LIFT_OK;
+}
+
+static lift::Exch make_exch(void *const *peers, int rank, int world, uint64_t epoch, int64_t cap) {
+    lift::Exch e;
+    e.peers = reinterpret_cast<char *const *>(peers);
+    e.rank = rank;
+    e.world = world;
+    e.epoch = epoch;
+    e.cap = cap;
+    return e;
+}
+
+int lift_dot_allreduce(int64_t n, const float *x, const float *y, float *result, void *workspace,
+                       size_t workspace_bytes, void *const *peers, int rank, int world, uint64_t epoch,
+                       lift_stream_t stream) {
+    int st = check_group(peers, rank, world, epoch);
+    if (st != LIFT_OK) return st;
+    if (!size_ok(n, 1)) return LIFT_ERR_BAD_SIZE;
+    if (result == nullptr) return LIFT_ERR_NULL_PTR;
+    if (n > 0 && (x == nullptr || y == nullptr)) return LIFT_ERR_NULL_PTR;
+    if (mis4(result) || (n > 0 && (mis4(x) || mis4(y)))) return LIFT_ERR_MISALIGNED;
+    if (workspace == nullptr || workspace_bytes < lift_dot_workspace_bytes(n) ||
+        (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const Range rr = rng(result, 4), rw = rng(workspace, workspace_bytes);
+    const Range rx = rng(x, (uint64_t)n * 4), ry = rng(y, (uint64_t)n * 4);
+    if (overlap(rr, rx) || overlap(rr, ry) || overlap(rr, rw) || overlap(rw, rx) || overlap(rw, ry))
+        return LIFT_ERR_ALIAS;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    return cuda_status(lift::launch_dot(d, n, x, y, result, workspace, (cudaStream_t)stream,
+                                        make_exch(peers, rank, world, epoch, lift::kMaxWorld)));
+}
+
+static int gather_common(int nmat, int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B,
+                         const float *x, int64_t row0, int64_t m_total, float *y, void *workspace,
+                         size_t workspace_bytes, void *const *peers, int rank, int world, uint64_t epoch,
+                         lift_stream_t stream) {
+    int st = check_group(peers, rank, world, epoch);
+    if (st != LIFT_OK) return st;
+    if (!size_ok(m, n) || !size_ok(m_total, 1) || row0 < 0 || row0 + m > m_total) return LIFT_ERR_BAD_SIZE;
+    if (m_total > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
+    if (m > 0 && n > 0 && (A == nullptr || x == nullptr || (nmat == 2 && B == nullptr))) return LIFT_ERR_NULL_PTR;
+    if ((m_total > 0 && mis4(y)) || (m > 0 && n > 0 && (mis4(A) || mis4(x) || (nmat == 2 && mis4(B)))))
+        return LIFT_ERR_MISALIGNED;
+    if (workspace == nullptr || workspace_bytes < 16 || (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const Range ry = rng(y, (uint64_t)m_total * 4), rw = rng(workspace, workspace_bytes);
+    const uint64_t mat = (uint64_t)m * (uint64_t)n * 4;
+    if (overlap(ry, rng(A, mat)) || overlap(ry, rng(x, (uint64_t)n * 4)) || (nmat == 2 && overlap(ry, rng(B, mat))) ||
+        overlap(ry, rw))
+        return LIFT_ERR_ALIAS;
+    if (m_total == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    lift::GemvArgs g;
+    g.nmat = nmat;
+    g.m = m;
+    g.n = n;
+    g.lda = n;
+    g.A = A;
+    g.B = B;
+    g.x = x;
+    g.y = y;
+    g.alpha = alpha;
+    g.beta = beta;
+    g.epi = nmat == 2 ? lift::kEpiSum2 : lift::kEpiStore;
+    g.ex = make_exch(peers, rank, world, epoch, m_total);
+    g.row0 = row0;
+    g.m_total = m_total;
+    g.ticket = static_cast<unsigned int *>(workspace);
+    return cuda_status(lift::launch_gemv(d, g, lift::GemvConfig{}, (cudaStream_t)stream));
+}
+
+int lift_gemv_allgather(int64_t m, int64_t n, const float *A, const float *x, int64_t row0, int64_t m_total,
+                        float *y, void *workspace, size_t workspace_bytes, void *const *peers, int rank, int world,
+                        uint64_t epoch, lift_stream_t stream) {
+    return gather_common(1, m, n, 1.f, A, 0.f, nullptr, x, row0, m_total, y, workspace, workspace_bytes, peers, rank,
+                         world, epoch, stream);
+}
+
+int lift_gesummv_allgather(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B,
+                           const float *x, int64_t row0, int64_t m_total, float *y, void *workspace,
+                           size_t workspace_bytes, void *const *peers, int rank, int world, uint64_t epoch,
+                           lift_stream_t stream) {
+    return gather_common(2, m, n, alpha, A, beta, B, x, row0, m_total, y, workspace, workspace_bytes, peers, rank,
+                         world, epoch, stream);
+}
+
+int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
+                     size_t workspace_bytes, void *const *peers, int rank, int world, int dst, uint64_t epoch,
+                     int blocks, lift_stream_t stream) {
+    int st = check_group(peers, rank, world, epoch);
+    if (st != LIFT_OK) return st;
+    if (dst < -1 || dst >= world || blocks < 0) return LIFT_ERR_BAD_SIZE;
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    const bool aligned = ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
+                           reinterpret_cast<uintptr_t>(y)) & 15) == 0;
+    if (n > 0 && !lift::atax_fused_preferred(m > 0 ? m : 1, n, aligned)) return LIFT_ERR_BAD_SIZE;
+    if (n > 0 && (y == nullptr || x == nullptr || (m > 0 && A == nullptr))) return LIFT_ERR_NULL_PTR;
+    if (workspace == nullptr || workspace_bytes < lift_atax_workspace_bytes(m, n) ||
+        (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const uint64_t mat = (uint64_t)m * (uint64_t)n * 4;
+    const Range ry = rng(y, (uint64_t)n * 4), rw = rng(workspace, workspace_bytes);
+    const Range rA = rng(A, mat), rx = rng(x, (uint64_t)n * 4);
+    if (overlap(ry, rA) || overlap(ry, rx) || overlap(ry, rw) || overlap(rw, rA) || overlap(rw, rx))
+        return LIFT_ERR_ALIAS;
+    if (n == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    return cuda_status(lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream,
+                                               make_exch(peers, rank, world, epoch, (int64_t)world * n), dst,
+                                               blocks));
 }
 
 const char *lift_strerror(int status) {

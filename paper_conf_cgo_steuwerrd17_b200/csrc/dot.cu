@@ -14,6 +14,7 @@
 // mapWrg over chunks (Fig. 7 l.7-8 = L954-955) becomes a persistent
 // grid-stride loop over a grid sized from the SM count.
 #include "common.cuh"
+#include "exchange.cuh"
 #include "launch.h"
 
 namespace lift {
@@ -36,7 +37,7 @@ __device__ __forceinline__ float block_sum(float v, float *red) {
 template <int TPB, int U, bool VEC>
 __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict__ x, const float *__restrict__ y,
                                              float *__restrict__ result, float *__restrict__ partials,
-                                             unsigned int *__restrict__ ticket) {
+                                             unsigned int *__restrict__ ticket, Exch ex) {
     __shared__ float red[TPB / kWarp];
     __shared__ bool am_last;
     const int64_t stride = (int64_t)gridDim.x * TPB;
@@ -107,13 +108,27 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
     __syncthreads();  // red[] reuse
     float tot = block_sum<TPB, U>(p, red);
     if (threadIdx.x == 0) {
-        *result = tot;
         *ticket = 0u;  // re-arm for the next launch on this workspace
+        if (ex.world == 0) {
+            *result = tot;
+        } else {
+            // fused all-reduce (NEXT-2): this rank's partial into slot `rank` of every
+            // rank's exchange area, publish, wait for all ranks, then every rank sums
+            // the slots in rank order: bitwise identical results on all ranks
+            for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex)[ex.rank] = tot;
+            __threadfence_system();
+            exch_signal(ex, -1);
+            exch_wait_all(ex);
+            const float *d = exch_data(ex.peers[ex.rank], ex);
+            float sum = 0.f;
+            for (int r = 0; r < ex.world; ++r) sum = __fadd_rn(sum, ld_volatile(d + r));
+            *result = sum;
+        }
     }
 }
 
 cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
-                       void *workspace, cudaStream_t s) {
+                       void *workspace, cudaStream_t s, Exch ex) {
     // B200 read sweep (tools/readbw.cu, profiles/r01j_readbw.txt): 256-thread blocks with
     // U = 4 float4 pairs in flight per thread and TWO waves of blocks stream fastest
     // (7.48 TB/s vs 7.39 for 512 threads / one wave); later blocks fill the tail.
@@ -135,9 +150,9 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;
     int blocks = (int)(want < 1 ? 1 : (want > cap ? cap : want));
     if (vec)
-        k_dot<TPB, U, true><<<blocks, TPB, 0, s>>>(n, x, y, result, partials, ticket);
+        k_dot<TPB, U, true><<<blocks, TPB, 0, s>>>(n, x, y, result, partials, ticket, ex);
     else
-        k_dot<TPB, U, false><<<blocks, TPB, 0, s>>>(n, x, y, result, partials, ticket);
+        k_dot<TPB, U, false><<<blocks, TPB, 0, s>>>(n, x, y, result, partials, ticket, ex);
     return cudaGetLastError();
 }
 

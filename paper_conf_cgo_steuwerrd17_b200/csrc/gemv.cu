@@ -22,6 +22,7 @@
 // row is the pairwise tree over the 8 slices.  A block row group of WPR warps
 // computes 8/WPR slices per warp, so every WPR gives the same bits.
 #include "common.cuh"
+#include "exchange.cuh"
 #include "launch.h"
 
 namespace lift {
@@ -66,7 +67,8 @@ template <int NMAT, int VEC, int WPR, int RG, bool XSMEM, int LB>
 __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, int64_t lda,
                                                         const float *__restrict__ A, const float *__restrict__ B,
                                                         const float *__restrict__ x, float *__restrict__ y,
-                                                        float alpha, float beta, int epi) {
+                                                        float alpha, float beta, int epi, Exch ex, int64_t row0,
+                                                        int64_t m_total, unsigned int *ticket) {
     using V = Vec<VEC>;
     using T = typename V::T;
     constexpr int KQ = kSlices / WPR;                                 // slices per warp
@@ -212,14 +214,20 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
                     buf ^= 1;
                 }
                 if (writer) {
+                    float val;
                     if constexpr (NMAT == 1) {
                         if (epi == kEpiStore)
-                            y[row] = s[0];
+                            val = s[0];
                         else  // kEpiAxpby (BLAS: y is not read when beta == 0)
-                            y[row] = beta == 0.f ? __fmul_rn(alpha, s[0])
-                                                 : __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, y[row]));
+                            val = beta == 0.f ? __fmul_rn(alpha, s[0])
+                                              : __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, y[row]));
                     } else {
-                        y[row] = __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, s[1]));
+                        val = __fadd_rn(__fmul_rn(alpha, s[0]), __fmul_rn(beta, s[1]));
+                    }
+                    if (ex.world == 0) {
+                        y[row] = val;
+                    } else {  // fused all-gather (NEXT-2): the row goes straight to every rank
+                        for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex)[row0 + row] = val;
                     }
                 }
                 if (nrow >= m) break;
@@ -237,6 +245,26 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     if constexpr (XSMEM) {
         // a row group that received no row must still retire the bulk copy
         if (x_pending) stage_wait(bar);
+    }
+    if (ex.world > 0) {
+        // all-gather completion: the last block of this rank publishes to every rank,
+        // waits for every rank, then copies the gathered y out of the exchange area
+        __shared__ int am_last;
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            __threadfence_system();  // this block's remote row stores are visible system-wide
+            am_last = atomicAdd(ticket, 1u) == gridDim.x - 1;
+        }
+        __syncthreads();
+        if (!am_last) return;
+        if (threadIdx.x == 0) {
+            *ticket = 0u;
+            exch_signal(ex, -1);
+            exch_wait_all(ex);
+        }
+        __syncthreads();
+        const float *src = exch_data(ex.peers[ex.rank], ex);
+        for (int64_t i = threadIdx.x; i < m_total; i += blockDim.x) y[i] = ld_volatile(src + i);
     }
 }
 
@@ -264,7 +292,8 @@ static cudaError_t run_gemv(const DeviceInfo &d, const GemvArgs &a, int blocks, 
     if (groups >= 32 * cap) cap *= 4;
     int64_t g = blocks > 0 ? blocks : (groups < cap ? groups : cap);
     if (g < 1) g = 1;
-    kern<<<(unsigned)g, threads, smem, s>>>(a.m, a.n, a.lda, a.A, a.B, a.x, a.y, a.alpha, a.beta, a.epi);
+    kern<<<(unsigned)g, threads, smem, s>>>(a.m, a.n, a.lda, a.A, a.B, a.x, a.y, a.alpha, a.beta, a.epi, a.ex, a.row0,
+                                            a.m_total, a.ticket);
     return cudaGetLastError();
 }
 

@@ -6,6 +6,8 @@
 #include <stddef.h>
 #include <stdint.h>
 
+#include "exchange.cuh"
+
 namespace lift {
 
 struct DeviceInfo {
@@ -24,7 +26,7 @@ cudaError_t device_info(DeviceInfo *out);
 constexpr int kDotMaxBlocks = 4096;
 constexpr size_t kDotTicketBytes = 16;
 cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
-                       void *workspace, cudaStream_t s);
+                       void *workspace, cudaStream_t s, Exch ex = Exch{});
 
 // ---- GEMV / GESUMMV ----------------------------------------------------------
 struct GemvConfig {
@@ -48,6 +50,11 @@ struct GemvArgs {
     float *y = nullptr;
     float alpha = 1.f, beta = 0.f;
     int epi = kEpiStore;
+    // fused all-gather (NEXT-2): rows go to every rank's exchange area at row0 + i;
+    // the last block waits for all ranks and copies the m_total gathered rows to y
+    Exch ex;
+    int64_t row0 = 0, m_total = 0;
+    unsigned int *ticket = nullptr;  // zeroed once; re-armed by every launch
 };
 cudaError_t launch_gemv(const DeviceInfo &d, const GemvArgs &a, GemvConfig cfg, cudaStream_t s);
 
@@ -64,7 +71,7 @@ size_t gemv_t_ws_bytes(int64_t m, int64_t n);
 cudaError_t launch_gemv_t(const DeviceInfo &d, int64_t m, int64_t n, int64_t lda, float alpha, const float *A,
                           const float *x, float beta, float *y, void *ws, cudaStream_t s);
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
-                              float *y, void *ws, cudaStream_t s);
+                              float *y, void *ws, cudaStream_t s, Exch ex = Exch{}, int dst = -1, int blocks = 0);
 
 // ---- Listing 1 in the paper's exact order (NEXT-3) ------------------------------
 cudaError_t launch_partial_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *z, bool fma,

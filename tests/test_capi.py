@@ -151,7 +151,9 @@ def test_python_binding_rejects_cpu_tensors():
 def test_ctypes_signatures_match_header_arity():
     import re
 
-    txt = open(_lib._build.INCLUDE + "/lift.h").read() + open(_lib._build.INCLUDE + "/lift_tuning.h").read()
+    import glob
+
+    txt = "".join(open(f).read() for f in sorted(glob.glob(_lib._build.INCLUDE + "/*.h")))
     txt = re.sub(r"/\*.*?\*/", "", txt, flags=re.S)
     for name, (_, args) in _lib.SIGNATURES.items():
         m = re.search(r"\b" + name + r"\s*\(([^)]*)\)", txt)
@@ -187,3 +189,23 @@ def test_sgemv_validation():
     assert L.lift_sgemv(0, 1, 4, 4, 1.0, A_, 4, X_, 0.0, Y_, None, 0, None) == WS
     assert L.lift_sgemv(0, 0, 4, 4, 1.0, A_, 8, X_, 0.0, A_ + 4 * 9, None, 0, None) == ALIAS
     assert L.lift_sgemv(0, 0, 0, 4, 1.0, None, 4, None, 0.0, None, None, 0, None) == OK
+
+
+def test_nvlink_validation():
+    peers = P * 400
+    ws = L.lift_dot_workspace_bytes(100)
+    assert L.lift_exchange_bytes(0, 0, 8) >= 1024 + 2 * 64 * 4
+    assert L.lift_exchange_bytes(1, 65536, 8) >= 2 * 65536 * 4
+    assert L.lift_exchange_bytes(2, 8192, 8) >= 2 * 8 * 8192 * 4
+    assert L.lift_exchange_bytes(3, 10, 8) == 0 and L.lift_exchange_bytes(0, 1, 65) == 0
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers, 0, 2, 0, None) == SIZE   # epoch 0
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers, 2, 2, 1, None) == SIZE   # rank >= world
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, None, 0, 2, 1, None) == NULL
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers + 4, 0, 2, 1, None) == MIS
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 95, 100, Y_, W_, 256, peers, 0, 2, 1, None) == SIZE  # rows past m_total
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, A_, W_, 256, peers, 0, 2, 1, None) == ALIAS
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, Y_, W_, 8, peers, 0, 2, 1, None) == WS
+    assert L.lift_gesummv_allgather(10, 4, 1.0, A_, 1.0, None, X_, 0, 10, Y_, W_, 256, peers, 0, 1, 1, None) == NULL
+    wsa = L.lift_atax_workspace_bytes(64, 512)
+    assert L.lift_atax_reduce(64, 512, A_, X_, Y_, W_, wsa, peers, 0, 2, 2, 1, 0, None) == SIZE      # dst >= world
+    assert L.lift_atax_reduce(64, 510, A_, X_, Y_, W_, wsa, peers, 0, 2, 0, 1, 0, None) == SIZE     # n % 4

@@ -1,0 +1,108 @@
+"""Collectives fused into the kernels (include/lift_nvlink.h, NEXT-2), run as
+`world` simulated ranks on ONE GPU: every rank's exchange area is a separate
+HBM allocation, all ranks share one peer table, and each rank's kernel is
+launched on its own stream so the ranks run concurrently — the same kernels
+and the same flag / epoch / parity protocol a multi-GPU run uses over NVLink
+(only the transport differs: same-device stores instead of NVLink stores).
+"""
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import synth
+import paper_conf_cgo_steuwerrd17_b200 as lift
+from paper_conf_cgo_steuwerrd17_b200 import nvlink
+from paper_conf_cgo_steuwerrd17_b200.shard import partition_rows
+
+pytestmark = [pytest.mark.gpu, pytest.mark.timeout(300)]
+
+
+def run_ranks(world, fn):
+    """fn(rank) launches rank's work on the current stream; all ranks concurrently."""
+    streams = [torch.cuda.Stream() for _ in range(world)]
+    outs = [None] * world
+    torch.cuda.synchronize()
+    for r in range(world):
+        with torch.cuda.stream(streams[r]):
+            outs[r] = fn(r)
+    torch.cuda.synchronize()
+    return outs
+
+
+@pytest.mark.parametrize("world", [1, 2, 3, 4, 8])
+def test_dot_allreduce_sim(cuda_device, world):
+    n = (1 << 20) + 13
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    y = synth.torch_uniform(synth.SEED_Y, 0, n, device=cuda_device)
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_DOT, 0, world, cuda_device)
+    parts = [partition_rows(n, world, r) for r in range(world)]
+    ref, mag = oracle.dot(x.cpu().numpy(), y.cpu().numpy())
+    for it in range(3):  # successive epochs exercise the parity double buffer
+        outs = run_ranks(world, lambda r: nvlink.lift_dot_allreduce(x[parts[r][0]:parts[r][1]],
+                                                                    y[parts[r][0]:parts[r][1]], exs[r]))
+        vals = [o.item() for o in outs]
+        assert all(np.float32(v).view(np.uint32) == np.float32(vals[0]).view(np.uint32) for v in vals)
+        ok, margin = oracle.within_tol([vals[0]], [ref], [mag])
+        assert ok, margin
+        # exactly the rank-order sum of the per-rank dots
+        per = [lift.lift_dot(x[a:b], y[a:b]).item() for a, b in parts]
+        s = np.float32(0)
+        for v in per:
+            s = np.float32(s + np.float32(v))
+        assert np.float32(vals[0]) == s
+
+
+@pytest.mark.parametrize("world", [2, 3, 4, 8])
+@pytest.mark.parametrize("op", ["gemv", "gesummv"])
+def test_gemv_allgather_sim(cuda_device, world, op):
+    m, n = 1000, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    B = synth.torch_matrix_rows(synth.SEED_B, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    full = lift.lift_gemv(A, x) if op == "gemv" else lift.lift_gesummv(1.5, A, 1.2, B, x)
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_GATHER, m, world, cuda_device)
+    parts = [partition_rows(m, world, r) for r in range(world)]
+    for it in range(3):
+        outs = run_ranks(world, lambda r: nvlink.lift_gemv_allgather(
+            A[parts[r][0]:parts[r][1]], x, parts[r][0], m, exs[r],
+            B=None if op == "gemv" else B[parts[r][0]:parts[r][1]], alpha=1.5, beta=1.2))
+        for r in range(world):
+            assert torch.equal(outs[r], full), (r, it)  # bitwise: canonical row order
+
+
+@pytest.mark.parametrize("world", [1, 2, 4])
+@pytest.mark.parametrize("dst", [-1, 0, 1])
+def test_atax_reduce_sim(cuda_device, world, dst):
+    if dst >= world:
+        pytest.skip("dst outside the group")
+    m, n = 3000, 4096
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
+    parts = [partition_rows(m, world, r) for r in range(world)]
+    blocks = 148 // world  # every rank's blocks co-resident on the one GPU
+    for it in range(2):
+        outs = run_ranks(world, lambda r: nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], x, exs[r], dst=dst,
+                                                                  blocks=blocks))
+        dsts = range(world) if dst < 0 else [dst]
+        for r in dsts:
+            ok, margin = oracle.within_tol(outs[r].cpu().numpy(), ref, mag)
+            assert ok, (r, margin)
+            assert torch.equal(outs[r], outs[dsts[0]])
+
+
+def test_atax_reduce_rank_with_no_rows(cuda_device):
+    world, n = 3, 512
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, 2, device=cuda_device)  # 2 rows over 3 ranks
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
+    parts = [partition_rows(2, world, r) for r in range(world)]
+    assert parts[0][1] - parts[0][0] == 0
+    outs = run_ranks(world, lambda r: nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], x, exs[r], dst=-1,
+                                                              blocks=8))
+    for r in range(world):
+        ok, margin = oracle.within_tol(outs[r].cpu().numpy(), ref, mag)
+        assert ok, margin
