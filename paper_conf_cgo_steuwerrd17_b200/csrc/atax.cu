@@ -602,6 +602,21 @@ static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const flo
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst);
 }
 
+cudaError_t preload_atax() {  // see preload_dot (dot.cu)
+    cudaFuncAttributes a;
+    cudaError_t e = cudaFuncGetAttributes(&a, k_atax_fused<1, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<4, 256, 8>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<1, 256, 8>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_colsum<4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_colsum<1>);
+    return e;
+}
+
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
                               void *ws, cudaStream_t s, Exch ex, int dst, int blocks) {
     if (n == 0) return cudaSuccess;

@@ -39,6 +39,11 @@ cudaError_t device_info(DeviceInfo *out) {
         if ((e = cudaDeviceGetAttribute(&t.regs_per_sm, cudaDevAttrMaxRegistersPerMultiprocessor, dev)) !=
             cudaSuccess)
             return e;
+        // eager load (lazy loading at a first launch waits for an idle device, which a
+        // kernel spinning on a peer's flag never allows)
+        if ((e = preload_dot()) != cudaSuccess || (e = preload_gemv()) != cudaSuccess ||
+            (e = preload_atax()) != cudaSuccess || (e = preload_listing1()) != cudaSuccess)
+            return e;
         d = t;
     }
     *out = d;

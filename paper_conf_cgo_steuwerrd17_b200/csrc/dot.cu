@@ -156,4 +156,14 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     return cudaGetLastError();
 }
 
+// Load every kernel of this unit now (CUDA's lazy loading would otherwise load a
+// kernel at its first launch, which waits for the device to go idle: a kernel
+// spinning on a peer's flag, as the fused collectives do, would never let it).
+cudaError_t preload_dot() {
+    cudaFuncAttributes a;
+    cudaError_t e = cudaFuncGetAttributes(&a, k_dot<256, 4, true>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_dot<256, 4, false>);
+    return e;
+}
+
 }  // namespace lift

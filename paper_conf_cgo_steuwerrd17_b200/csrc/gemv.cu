@@ -317,6 +317,38 @@ static cudaError_t dispatch_wpr(const DeviceInfo &d, int wpr, int rg, int lb, co
     return cudaErrorInvalidValue;
 }
 
+template <int NMAT, int VEC, bool XSMEM, int LB>
+static cudaError_t preload_set() {
+    cudaFuncAttributes a;
+    cudaError_t e = cudaSuccess;
+#define LIFT_PRELOAD(W, R) \
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_gemv<NMAT, VEC, W, R, XSMEM, LB>);
+    LIFT_PRELOAD(8, 1)
+    LIFT_PRELOAD(8, 2)
+    LIFT_PRELOAD(4, 2)
+    LIFT_PRELOAD(4, 4)
+    LIFT_PRELOAD(2, 4)
+    LIFT_PRELOAD(2, 8)
+    LIFT_PRELOAD(1, 8)
+#undef LIFT_PRELOAD
+    return e;
+}
+
+cudaError_t preload_gemv() {  // see preload_dot (dot.cu)
+    cudaError_t e = preload_set<1, 4, true, 4>();
+    if (e == cudaSuccess) e = preload_set<1, 4, true, 8>();
+    if (e == cudaSuccess) e = preload_set<1, 4, false, 4>();
+    if (e == cudaSuccess) e = preload_set<1, 4, false, 8>();
+    if (e == cudaSuccess) e = preload_set<2, 4, true, 4>();
+    if (e == cudaSuccess) e = preload_set<2, 4, true, 8>();
+    if (e == cudaSuccess) e = preload_set<2, 4, false, 4>();
+    if (e == cudaSuccess) e = preload_set<2, 4, false, 8>();
+    cudaFuncAttributes a;
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_gemv<1, 1, 1, 8, false, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_gemv<2, 1, 1, 8, false, 4>);
+    return e;
+}
+
 cudaError_t launch_gemv(const DeviceInfo &d, const GemvArgs &a, GemvConfig cfg, cudaStream_t s) {
     const int64_t m = a.m, n = a.n;
     if (m == 0) return cudaSuccess;

@@ -19,8 +19,13 @@ struct DeviceInfo {
     int regs_per_sm = 0;      // 65536
 };
 
-// Cached per device; thread-safe after the first call per device.
+// Cached per device; thread-safe after the first call per device.  The first
+// call on a device also loads every kernel of the library (preload_*).
 cudaError_t device_info(DeviceInfo *out);
+cudaError_t preload_dot();
+cudaError_t preload_gemv();
+cudaError_t preload_atax();
+cudaError_t preload_listing1();
 
 // ---- dot -------------------------------------------------------------------
 constexpr int kDotMaxBlocks = 4096;

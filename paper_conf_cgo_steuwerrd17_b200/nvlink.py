@@ -68,8 +68,25 @@ class ExchangeArea:
         return self.epoch
 
 
-def lift_dot_allreduce(x: torch.Tensor, y: torch.Tensor, ex: ExchangeArea, out: torch.Tensor | None = None):
-    """Sum over ranks of dot(x_r, y_r); the same bits on every rank."""
+def workspace_bytes(op: str, m: int = 0, n: int = 0) -> int:
+    """Workspace bytes of one call (allocate zeroed, reuse across calls)."""
+    L = lib()
+    if op == "dot":
+        return L.lift_dot_workspace_bytes(n)
+    if op in ("gemv", "gesummv"):
+        return 256
+    if op == "atax":
+        return L.lift_atax_workspace_bytes(m, n)
+    raise ValueError(op)
+
+
+def lift_dot_allreduce(x: torch.Tensor, y: torch.Tensor, ex: ExchangeArea, out: torch.Tensor | None = None,
+                       workspace: torch.Tensor | None = None):
+    """Sum over ranks of dot(x_r, y_r); the same bits on every rank.
+
+    Pass `out` and `workspace` (zeroed uint8) when ranks share one device:
+    allocating inside the call may synchronise the device while a peer rank's
+    kernel is waiting for this one."""
     _check_tensor(x, "x", 1)
     _check_tensor(y, "y", 1)
     dev = _same_device(x, y)
@@ -79,7 +96,8 @@ def lift_dot_allreduce(x: torch.Tensor, y: torch.Tensor, ex: ExchangeArea, out: 
     L = lib()
     n = x.numel()
     with torch.cuda.device(dev):
-        ws = _workspace(f"dotar{ex.rank}", dev, L.lift_dot_workspace_bytes(n), zero=True)
+        ws = workspace if workspace is not None else _workspace(f"dotar{ex.rank}", dev,
+                                                                L.lift_dot_workspace_bytes(n), zero=True)
         check(L.lift_dot_allreduce(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
                                    ex.peers.data_ptr(), ex.rank, ex.world, ex.next_epoch(), _stream(dev)))
     return out
@@ -87,7 +105,7 @@ def lift_dot_allreduce(x: torch.Tensor, y: torch.Tensor, ex: ExchangeArea, out: 
 
 def lift_gemv_allgather(A: torch.Tensor, x: torch.Tensor, row0: int, m_total: int, ex: ExchangeArea,
                         out: torch.Tensor | None = None, B: torch.Tensor | None = None, alpha: float = 1.0,
-                        beta: float = 0.0):
+                        beta: float = 0.0, workspace: torch.Tensor | None = None):
     """Rows [row0, row0 + A.shape[0]) computed here; the full y on every rank.
     With B given: GESUMMV (alpha A x + beta B x)."""
     _check_tensor(A, "A", 2)
@@ -99,7 +117,7 @@ def lift_gemv_allgather(A: torch.Tensor, x: torch.Tensor, row0: int, m_total: in
         out = torch.empty(m_total, dtype=torch.float32, device=dev)
     L = lib()
     with torch.cuda.device(dev):
-        ws = _workspace(f"gather{ex.rank}", dev, 256, zero=True)
+        ws = workspace if workspace is not None else _workspace(f"gather{ex.rank}", dev, 256, zero=True)
         if B is None:
             st = L.lift_gemv_allgather(m, n, A.data_ptr(), x.data_ptr(), row0, m_total, out.data_ptr(), ws.data_ptr(),
                                        ws.numel(), ex.peers.data_ptr(), ex.rank, ex.world, ex.next_epoch(),
@@ -114,7 +132,7 @@ def lift_gemv_allgather(A: torch.Tensor, x: torch.Tensor, row0: int, m_total: in
 
 
 def lift_atax_reduce(A: torch.Tensor, x: torch.Tensor, ex: ExchangeArea, dst: int = -1,
-                     out: torch.Tensor | None = None, blocks: int = 0):
+                     out: torch.Tensor | None = None, blocks: int = 0, workspace: torch.Tensor | None = None):
     """y = sum over ranks of A_r^T (A_r x) on `dst` (-1: every rank)."""
     _check_tensor(A, "A", 2)
     _check_tensor(x, "x", 1)
@@ -125,7 +143,8 @@ def lift_atax_reduce(A: torch.Tensor, x: torch.Tensor, ex: ExchangeArea, dst: in
         out = torch.empty(n, dtype=torch.float32, device=dev)
     L = lib()
     with torch.cuda.device(dev):
-        ws = _workspace(f"ataxr{ex.rank}", dev, L.lift_atax_workspace_bytes(m, n), zero=True)
+        ws = workspace if workspace is not None else _workspace(f"ataxr{ex.rank}", dev,
+                                                                L.lift_atax_workspace_bytes(m, n), zero=True)
         check(L.lift_atax_reduce(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
                                  ex.peers.data_ptr(), ex.rank, ex.world, dst, ex.next_epoch(), blocks, _stream(dev)))
     return out

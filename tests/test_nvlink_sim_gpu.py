@@ -19,7 +19,9 @@ pytestmark = [pytest.mark.gpu, pytest.mark.timeout(300)]
 
 
 def run_ranks(world, fn):
-    """fn(rank) launches rank's work on the current stream; all ranks concurrently."""
+    """fn(rank) launches rank's work on the current stream; all ranks concurrently.
+    Everything fn touches must be allocated beforehand: an allocation inside the
+    launch loop may synchronise the device while rank 0 waits for rank 1."""
     streams = [torch.cuda.Stream() for _ in range(world)]
     outs = [None] * world
     torch.cuda.synchronize()
@@ -30,6 +32,13 @@ def run_ranks(world, fn):
     return outs
 
 
+def prealloc(world, op, m, n, out_shape, device):
+    ws = [torch.zeros(nvlink.workspace_bytes(op, m, n), dtype=torch.uint8, device=device) for _ in range(world)]
+    outs = [torch.empty(out_shape, dtype=torch.float32, device=device) for _ in range(world)]
+    torch.cuda.synchronize()
+    return ws, outs
+
+
 @pytest.mark.parametrize("world", [1, 2, 3, 4, 8])
 def test_dot_allreduce_sim(cuda_device, world):
     n = (1 << 20) + 13
@@ -38,9 +47,11 @@ def test_dot_allreduce_sim(cuda_device, world):
     exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_DOT, 0, world, cuda_device)
     parts = [partition_rows(n, world, r) for r in range(world)]
     ref, mag = oracle.dot(x.cpu().numpy(), y.cpu().numpy())
+    ws, res = prealloc(world, "dot", 0, n, (), cuda_device)
     for it in range(3):  # successive epochs exercise the parity double buffer
         outs = run_ranks(world, lambda r: nvlink.lift_dot_allreduce(x[parts[r][0]:parts[r][1]],
-                                                                    y[parts[r][0]:parts[r][1]], exs[r]))
+                                                                    y[parts[r][0]:parts[r][1]], exs[r],
+                                                                    out=res[r], workspace=ws[r]))
         vals = [o.item() for o in outs]
         assert all(np.float32(v).view(np.uint32) == np.float32(vals[0]).view(np.uint32) for v in vals)
         ok, margin = oracle.within_tol([vals[0]], [ref], [mag])
@@ -63,9 +74,10 @@ def test_gemv_allgather_sim(cuda_device, world, op):
     full = lift.lift_gemv(A, x) if op == "gemv" else lift.lift_gesummv(1.5, A, 1.2, B, x)
     exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_GATHER, m, world, cuda_device)
     parts = [partition_rows(m, world, r) for r in range(world)]
+    ws, res = prealloc(world, op, m, n, (m,), cuda_device)
     for it in range(3):
         outs = run_ranks(world, lambda r: nvlink.lift_gemv_allgather(
-            A[parts[r][0]:parts[r][1]], x, parts[r][0], m, exs[r],
+            A[parts[r][0]:parts[r][1]], x, parts[r][0], m, exs[r], out=res[r], workspace=ws[r],
             B=None if op == "gemv" else B[parts[r][0]:parts[r][1]], alpha=1.5, beta=1.2))
         for r in range(world):
             assert torch.equal(outs[r], full), (r, it)  # bitwise: canonical row order
@@ -83,9 +95,10 @@ def test_atax_reduce_sim(cuda_device, world, dst):
     exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
     parts = [partition_rows(m, world, r) for r in range(world)]
     blocks = 148 // world  # every rank's blocks co-resident on the one GPU
+    ws, res = prealloc(world, "atax", m, n, (n,), cuda_device)
     for it in range(2):
         outs = run_ranks(world, lambda r: nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], x, exs[r], dst=dst,
-                                                                  blocks=blocks))
+                                                                  blocks=blocks, out=res[r], workspace=ws[r]))
         dsts = range(world) if dst < 0 else [dst]
         for r in dsts:
             ok, margin = oracle.within_tol(outs[r].cpu().numpy(), ref, mag)
@@ -101,8 +114,9 @@ def test_atax_reduce_rank_with_no_rows(cuda_device):
     exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
     parts = [partition_rows(2, world, r) for r in range(world)]
     assert parts[0][1] - parts[0][0] == 0
+    ws, res = prealloc(world, "atax", 2, n, (n,), cuda_device)
     outs = run_ranks(world, lambda r: nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], x, exs[r], dst=-1,
-                                                              blocks=8))
+                                                              blocks=8, out=res[r], workspace=ws[r]))
     for r in range(world):
         ok, margin = oracle.within_tol(outs[r].cpu().numpy(), ref, mag)
         assert ok, margin
