@@ -309,9 +309,21 @@ def run_ours(args) -> None:
         bufs[name] = b
     torch.cuda.synchronize()
 
+    fused = distributed and args.collectives == "fused"
+    fg = shard.FusedGroup() if fused else None
+
     def run_op(name, op, shp):
-        """local compute (our kernels) then the op's one collective (N > 1)."""
+        """local compute (our kernels) then the op's one collective (N > 1): NCCL, or
+        fused into the kernel over NVLink peer stores (--collectives fused)."""
         b = bufs[name]
+        if fused:
+            if op == "dot":
+                return shard.dot_fused(b["x"], b["y"], fg, out=b["out"])
+            if op == "gemv":
+                return shard.gemv_fused(b["A"], b["x"], shp["m"], fg, out=b["y"])
+            if op == "gesummv":
+                return shard.gesummv_fused(ALPHA, b["A"], BETA, b["B"], b["x"], shp["m"], fg, out=b["y"])
+            return shard.atax_fused(b["A"], b["x"], fg, dst=0, out=b["y"])
         if op == "dot":
             if distributed:
                 return shard.dot(b["x"], b["y"])
@@ -453,6 +465,7 @@ def run_ours(args) -> None:
             "scaling": "strong", "vs_baseline": None, "dtype": "f32",
             "data": "synthetic: seeded counter-based U[-1,1) fp32 generated in HBM (synth/); paper data sets not shipped",
             "config": {"workload": WORKLOAD_NAME, "parallelism": f"row-sharded x{world}" if world > 1 else "1 GPU",
+                       "collectives": (args.collectives if world > 1 else None),
                        "l2": "inputs larger than L2: each step streams ~25 GiB; every operand is evicted by the "
                              "following ops before reuse (no flush kernel in the timed region)",
                        "atax_algo": atax_algo, "alpha": ALPHA, "beta": BETA,
@@ -544,6 +557,9 @@ def main():
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline oracle timing")
     ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--eager", action="store_true", help="launch the timed steps eagerly instead of as a CUDA graph")
+    ap.add_argument("--collectives", choices=["nccl", "fused"], default="nccl",
+                    help="N > 1: NCCL collectives (default) or the collective fused into the kernels over "
+                         "NVLink symmetric memory (include/lift_nvlink.h)")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     args = ap.parse_args()
     if args.impl == "reference":

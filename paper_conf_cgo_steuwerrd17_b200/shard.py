@@ -135,3 +135,66 @@ def atax(A_loc: torch.Tensor, x: torch.Tensor, group=None, dst: int = 0, allredu
         return y
     dist.reduce(y, dst=dst, op=dist.ReduceOp.SUM, group=group)
     return y if dist.get_rank(group) == dst else None
+
+
+# ---------------------------------------------------------------------------
+# the same ops with the collective fused into the kernel (include/lift_nvlink.h)
+# ---------------------------------------------------------------------------
+class FusedGroup:
+    """Per-op exchange areas in torch symmetric memory (NVLink peer mappings).
+
+    ``FusedGroup(group)`` must be created collectively; each op/shape gets its
+    own area on first use (also a collective: every rank calls the same ops in
+    the same order, exactly as with NCCL).  For single-GPU tests pass
+    ``areas`` built with :meth:`nvlink.ExchangeArea.simulated`.
+    """
+
+    def __init__(self, group=None, areas: Optional[dict] = None):
+        self.group = group
+        self.areas = areas if areas is not None else {}
+
+    def area(self, kind: int, length: int):
+        from .nvlink import ExchangeArea
+
+        key = (kind, length)
+        if key not in self.areas:
+            self.areas[key] = ExchangeArea.symmetric(kind, length, self.group)
+        return self.areas[key]
+
+
+def dot_fused(x_loc: torch.Tensor, y_loc: torch.Tensor, fg: FusedGroup, out=None) -> torch.Tensor:
+    """dot with the all-reduce inside the kernel: identical bits on every rank."""
+    from .nvlink import EXCH_DOT, lift_dot_allreduce
+
+    return lift_dot_allreduce(x_loc, y_loc, fg.area(EXCH_DOT, 0), out=out)
+
+
+def gemv_fused(A_loc: torch.Tensor, x: torch.Tensor, m: int, fg: FusedGroup, row0: Optional[int] = None,
+               out=None) -> torch.Tensor:
+    """GEMV whose rows are stored straight into every rank's y (fused all-gather)."""
+    from .nvlink import EXCH_GATHER, lift_gemv_allgather
+
+    ex = fg.area(EXCH_GATHER, m)
+    if row0 is None:
+        row0 = partition_rows(m, ex.world, ex.rank)[0]
+    return lift_gemv_allgather(A_loc, x, row0, m, ex, out=out)
+
+
+def gesummv_fused(alpha: float, A_loc: torch.Tensor, beta: float, B_loc: torch.Tensor, x: torch.Tensor, m: int,
+                  fg: FusedGroup, row0: Optional[int] = None, out=None) -> torch.Tensor:
+    from .nvlink import EXCH_GATHER, lift_gemv_allgather
+
+    ex = fg.area(EXCH_GATHER, m)
+    if row0 is None:
+        row0 = partition_rows(m, ex.world, ex.rank)[0]
+    return lift_gemv_allgather(A_loc, x, row0, m, ex, out=out, B=B_loc, alpha=alpha, beta=beta)
+
+
+def atax_fused(A_loc: torch.Tensor, x: torch.Tensor, fg: FusedGroup, dst: int = 0, allreduce: bool = False,
+               out=None) -> Optional[torch.Tensor]:
+    """ATAX whose partial A_r^T (A_r x) is reduced over ranks inside the kernel."""
+    from .nvlink import EXCH_REDUCE, lift_atax_reduce
+
+    ex = fg.area(EXCH_REDUCE, x.numel())
+    y = lift_atax_reduce(A_loc, x, ex, dst=-1 if allreduce else dst, out=out)
+    return y if (allreduce or ex.rank == dst) else None
