@@ -278,11 +278,16 @@ def run_ours(args) -> None:
     local_rank = int(os.environ.get("LOCAL_RANK", "0"))
     if args.gpus != world and world > 1:
         raise SystemExit(f"--gpus {args.gpus} but WORLD_SIZE={world}")
+    if args.test_one_device:  # test harness: every rank on cuda:0 (numbers meaningless)
+        local_rank = 0
     torch.cuda.set_device(local_rank)
     dev = torch.device("cuda", local_rank)
     distributed = world > 1
     if distributed:
-        dist.init_process_group("nccl", device_id=dev)
+        if args.test_backend == "nccl":
+            dist.init_process_group("nccl", device_id=dev)
+        else:
+            dist.init_process_group(args.test_backend)
     if args.warmup < 3:
         raise SystemExit("--warmup must be >= 3")
 
@@ -355,7 +360,7 @@ def run_ours(args) -> None:
 
     def barrier():
         if distributed:
-            dist.barrier(device_ids=[local_rank])
+            dist.barrier(device_ids=[local_rank]) if args.test_backend == "nccl" else dist.barrier()
         torch.cuda.synchronize()
 
     # 1 GPU: the K timed steps are one CUDA graph (no host launch gaps between the
@@ -476,7 +481,7 @@ def run_ours(args) -> None:
         }
         print(json.dumps(line), flush=True)
     if distributed:
-        dist.barrier(device_ids=[local_rank])
+        dist.barrier(device_ids=[local_rank]) if args.test_backend == "nccl" else dist.barrier()
         dist.destroy_process_group()
 
 
@@ -557,11 +562,19 @@ def main():
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline oracle timing")
     ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--eager", action="store_true", help="launch the timed steps eagerly instead of as a CUDA graph")
+    ap.add_argument("--test-backend", default="nccl", help=argparse.SUPPRESS)  # tests: gloo with CUDA tensors
+    ap.add_argument("--test-one-device", action="store_true", help=argparse.SUPPRESS)  # tests: all ranks on cuda:0
+    ap.add_argument("--scale", type=float, default=1.0, help=argparse.SUPPRESS)  # tests: shrink the workload
     ap.add_argument("--collectives", choices=["nccl", "fused"], default="nccl",
                     help="N > 1: NCCL collectives (default) or the collective fused into the kernels over "
                          "NVLink symmetric memory (include/lift_nvlink.h)")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     args = ap.parse_args()
+    if args.scale != 1.0:  # test harness only: shrink rows / elements, keep the shapes' columns
+        global WORKLOAD
+        WORKLOAD = [(nm, op, ({"n": max(4, int(shp["n"] * args.scale) // 4 * 4)} if op == "dot" else
+                              {"m": max(1, int(shp["m"] * args.scale)), "n": shp["n"]}), cfg)
+                    for nm, op, shp, cfg in WORKLOAD]
     if args.impl == "reference":
         run_reference(args)
     else:
