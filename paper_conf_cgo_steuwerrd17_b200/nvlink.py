@@ -56,6 +56,60 @@ class ExchangeArea:
         return cls(kind, length, area, peers, rank, world)
 
     @classmethod
+    def ipc(cls, kind: int, length: int, group=None) -> "ExchangeArea":
+        """This rank's area from cudaMalloc, shared with CUDA IPC handles (collective).
+
+        The transport for ranks that torch symmetric memory refuses (e.g. several
+        processes on one GPU); across GPUs the opened handles map the peers' HBM
+        over NVLink (cudaIpcMemLazyEnablePeerAccess)."""
+        import torch.distributed as dist
+        from cuda.bindings import runtime as rt
+
+        def ok(res):
+            err = res[0] if isinstance(res, tuple) else res
+            if int(err) != 0:
+                raise RuntimeError(f"CUDA runtime error {err}")
+            return res[1] if isinstance(res, tuple) and len(res) > 1 else None
+
+        world, rank = dist.get_world_size(group), dist.get_rank(group)
+        dev_index = torch.cuda.current_device()
+        ok(rt.cudaSetDevice(dev_index))
+        nb = cls.nbytes(kind, length, world)
+        ptr = int(ok(rt.cudaMalloc(nb)))
+        ok(rt.cudaMemset(ptr, 0, nb))
+        ok(rt.cudaDeviceSynchronize())
+        handle = ok(rt.cudaIpcGetMemHandle(ptr))
+        mine = bytes(handle.reserved)
+        handles = [None] * world
+        dist.all_gather_object(handles, mine, group=group)
+        ptrs, opened = [], []
+        for r, hb in enumerate(handles):
+            if r == rank:
+                ptrs.append(ptr)
+                continue
+            h = rt.cudaIpcMemHandle_t()
+            h.reserved = hb
+            p = int(ok(rt.cudaIpcOpenMemHandle(h, rt.cudaIpcMemLazyEnablePeerAccess)))
+            ptrs.append(p)
+            opened.append(p)
+        peers = torch.tensor(ptrs, dtype=torch.int64, device=torch.device("cuda", dev_index))
+        torch.cuda.synchronize()
+        dist.barrier(group)
+        ex = cls(kind, length, None, peers, rank, world)
+        ex._ipc = (rt, ptr, opened)
+        return ex
+
+    def close(self) -> None:
+        """Release an IPC area (collective: peers must be done with it)."""
+        ipc = getattr(self, "_ipc", None)
+        if ipc is not None:
+            rt, ptr, opened = ipc
+            for p in opened:
+                rt.cudaIpcCloseMemHandle(p)
+            rt.cudaFree(ptr)
+            self._ipc = None
+
+    @classmethod
     def simulated(cls, kind: int, length: int, world: int, device) -> list["ExchangeArea"]:
         """`world` areas on one device, one peer table: rank r's view is element r."""
         nb = cls.nbytes(kind, length, world)

@@ -149,16 +149,26 @@ class FusedGroup:
     ``areas`` built with :meth:`nvlink.ExchangeArea.simulated`.
     """
 
-    def __init__(self, group=None, areas: Optional[dict] = None):
+    def __init__(self, group=None, areas: Optional[dict] = None, transport: str = "auto"):
         self.group = group
         self.areas = areas if areas is not None else {}
+        self.transport = transport  # "symm" | "ipc" | "auto" (symmetric memory, else CUDA IPC)
 
     def area(self, kind: int, length: int):
         from .nvlink import ExchangeArea
 
         key = (kind, length)
         if key not in self.areas:
-            self.areas[key] = ExchangeArea.symmetric(kind, length, self.group)
+            ex = None
+            if self.transport in ("auto", "symm"):
+                try:
+                    ex = ExchangeArea.symmetric(kind, length, self.group)
+                except RuntimeError:
+                    if self.transport == "symm":
+                        raise
+            if ex is None:  # both transports map the peers' HBM; IPC also works for ranks sharing a GPU
+                ex = ExchangeArea.ipc(kind, length, self.group)
+            self.areas[key] = ex
         return self.areas[key]
 
 
