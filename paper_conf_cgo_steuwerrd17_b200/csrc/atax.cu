@@ -439,6 +439,9 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     int it = 0, buf = 0;   // it = rows loaded so far
     int prow = 0;          // rows of the previous step (0: none)
     int64_t prev_r = r0;   // first row of the previous step
+    int slot = 0;          // ring slot of row `it` (it % nst), tracked without division
+    uint32_t phase = 0;    // its mbarrier phase parity ((it / nst) & 1)
+    int pslot = 0;         // ring slot of the previous step's first row
     float4 ap[CR][QC];     // the previous step's rows, kept for its rank-1 updates
 #pragma unroll
     for (int i = 0; i < CR; ++i)
@@ -451,7 +454,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
             for (int i = 0; i < prow; ++i) {
                 const int64_t rn = prev_r + i + nst;  // the row NST ahead reuses this slot
                 if (rn < r1) {
-                    const int st = (it - prow + i) % nst;
+                    const int st = pslot + i < nst ? pslot + i : pslot + i - nst;
                     mbar_arrive_expect_tx(full + st, row_bytes);
                     bulk_g2s(stage0 + (size_t)st * n, A + rn * n, row_bytes, full + st);
                 }
@@ -463,8 +466,9 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 #pragma unroll
             for (int i = 0; i < CR; ++i) {
                 if (i < rows) {
-                    const int st = (it + i) % nst;
-                    mbar_wait_parity(full + st, (uint32_t)(((it + i) / nst) & 1));
+                    const bool wrap = slot + i >= nst;
+                    const int st = wrap ? slot + i - nst : slot + i;
+                    mbar_wait_parity(full + st, wrap ? phase ^ 1u : phase);
                     const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)st * n);
 #pragma unroll
                     for (int q = 0; q < QC; ++q) {
@@ -524,6 +528,12 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         prow = rows;
         prev_r = r;
         it += rows;
+        pslot = slot;
+        slot += rows;
+        if (slot >= nst) {
+            slot -= nst;
+            phase ^= 1u;
+        }
     }
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
 #pragma unroll

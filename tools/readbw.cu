@@ -108,7 +108,7 @@ static void run(const char *name, K kern, int tpb, int64_t bytes, Args... args) 
     }
 }
 
-int main() {
+int main(int argc, char **argv) {
     const int64_t n = (int64_t)1 << 30;  // 4 GiB per array
     float *x, *y, *out;
     cudaMalloc(&x, n * 4);
@@ -116,8 +116,41 @@ int main() {
     cudaMalloc(&out, 64);
     cudaMemset(x, 0, n * 4);
     cudaMemset(y, 0, n * 4);
-    const int64_t bytes = 8 * n;
     const float4 *x4 = (const float4 *)x, *y4 = (const float4 *)y;
+    if (argc > 1) {
+        // size sweep: the practical read ceiling of a SINGLE launch of a given size
+        // (L2 flushed by reading 1 GiB of y before each timed launch)
+        for (int64_t bytes : {(int64_t)8 << 20, (int64_t)64 << 20, (int64_t)256 << 20, (int64_t)512 << 20,
+                              (int64_t)2 << 30, (int64_t)8 << 30}) {
+            const int64_t m = bytes / 8;  // elements per array
+            int sms = 0, per_sm = 0;
+            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k4<4, 0>, 256, 0);
+            for (int mult : {1, 2}) {
+                int64_t want = (m / 4 + 255) / 256;
+                int64_t grid = (int64_t)per_sm * sms * mult;
+                if (grid > want) grid = want;
+                float best = 1e30f;
+                cudaEvent_t a, b;
+                cudaEventCreate(&a);
+                cudaEventCreate(&b);
+                for (int it = 0; it < 7; ++it) {
+                    k4<4, 0><<<per_sm * sms, 256>>>((int64_t)1 << 28, (const float4 *)y, (const float4 *)y, out);
+                    cudaEventRecord(a);
+                    k4<4, 0><<<(int)grid, 256>>>(m / 4, x4, x4 + m / 4, out);
+                    cudaEventRecord(b);
+                    cudaEventSynchronize(b);
+                    float ms;
+                    cudaEventElapsedTime(&ms, a, b);
+                    if (it >= 2 && ms < best) best = ms;
+                }
+                printf("single launch %6lld MiB  grid %5lld (x%d)  %9.2f us  %7.1f GB/s\n", (long long)(bytes >> 20),
+                       (long long)grid, mult, best * 1e3, bytes / (best * 1e-3) / 1e9);
+            }
+        }
+        return 0;
+    }
+    const int64_t bytes = 8 * n;
     run("v4 na U4", k4<4, 0>, 512, bytes, n / 4, x4, y4, out);
     run("v4 na U4", k4<4, 0>, 256, bytes, n / 4, x4, y4, out);
     run("v4 na U8", k4<8, 0>, 256, bytes, n / 4, x4, y4, out);
