@@ -216,8 +216,20 @@ def cpu_baseline(min_seconds: float = 10.0) -> dict:
         if el >= min_seconds:
             break
     gbs = total * passes / el / 1e9
+    # BASELINE.json configs[0]: the 2^20-element dot "CPU oracle in milliseconds"
+    import oracle
+    import synth
+
+    xs, ys = synth.numpy_uniform(synth.SEED_X, 0, 1 << 20), synth.numpy_uniform(synth.SEED_Y, 0, 1 << 20)
+    oracle.dot(xs, ys)
+    ts = []
+    for _ in range(5):
+        t1 = time.perf_counter()
+        oracle.dot(xs, ys)
+        ts.append(time.perf_counter() - t1)
     return {"value": round(gbs, 3), "unit": "GB/s", "cores": th, "kind": "oracle",
-            "sample": desc + f"; {passes} passes in {el:.1f} s"}
+            "sample": desc + f"; {passes} passes in {el:.1f} s",
+            "configs0_dot_2^20_ms": round(1e3 * sorted(ts)[2], 3)}
 
 
 def run_reference(args) -> None:
