@@ -79,20 +79,23 @@ def main(tag, prefix):
         lines = [f"# ncu launch list of `python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu` ({tag});",
                  "# cold-cache, serialised per-launch times: compare SHARES of the step, not absolutes", ""]
         tot = collections.OrderedDict()
-        per_step = sum(1 for _ in k.values()) // 5  # 3 warm-up + 2 timed steps
+        # bench.py --steps 2 --warmup 3 launches: 3 eager warm-up steps, then the CUDA graph of
+        # the 2 timed steps replayed twice (upload, then timed), then the per-op breakdown
+        kps, warm, steps = 5, 3, 2
+        t0, t1 = (warm + steps) * kps, (warm + 2 * steps) * kps
         for i, d in k.items():
             t = d.get("gpu__time_duration.sum", 0.0)
             rd, wr = d.get("dram__bytes_read.sum", 0.0), d.get("dram__bytes_write.sum", 0.0)
             nm = d["name"].split("(")[0].replace("void ", "")
             lines.append(f"{i:>4} {nm:34s} grid {d['grid']:>14} {t / 1e3:10.2f} us  dram {(rd + wr) / 1e6:10.2f} MB"
                          f"  {(rd + wr) / t if t else 0:8.1f} GB/s")
-            if int(i) >= 3 * per_step:  # the timed steps only
+            if t0 <= int(i) < t1:  # the timed steps only
                 a = tot.setdefault(nm, [0.0, 0.0, 0])
                 a[0] += t
                 a[1] += rd + wr
                 a[2] += 1
         s = sum(v[0] for v in tot.values()) or 1
-        lines += ["", "per-kernel share of the timed steps (ncu time):"]
+        lines += ["", f"per-kernel share of the timed steps (launches {t0}..{t1 - 1}, ncu time):"]
         for nm, (t, b, c) in sorted(tot.items(), key=lambda kv: -kv[1][0]):
             lines.append(f"  {nm:34s} launches {c:3d}  share {100 * t / s:6.2f}%  avg {t / c / 1e3:10.2f} us  "
                          f"dram/launch {b / c / 1e6:10.2f} MB")
