@@ -589,6 +589,17 @@ def run_e2e(args, bufs, run_op, dev, distributed, world, step_bytes):
     def e2e_step():
         for name, op, shp, _ in WORKLOAD:
             b, hb = bufs[name], host[name]
+            if not distributed:
+                # 1 GPU: the C-ABI host entry points (include/lift_host.h) do the H2D copies,
+                # the kernels and the D2H copy of the result on the stream
+                import paper_conf_cgo_steuwerrd17_b200 as lift
+
+                hd = {k: v for k, v in hb.items() if k != "res"}
+                hd["out"] = hb["res"]
+                dv = {k: b[k] for k in hd if k != "out"}
+                dv["out"] = b["out" if op == "dot" else "y"]
+                lift.lift_host_call(op, hd, dv, alpha=ALPHA, beta=BETA)
+                continue
             for key, h in hb.items():
                 if key != "res":
                     b[key].copy_(h, non_blocking=True)
@@ -616,7 +627,9 @@ def run_e2e(args, bufs, run_op, dev, distributed, world, step_bytes):
     ms_step = ms / steps
     return {"value": round(step_bytes / (ms_step * 1e-3) / 1e9, 2), "unit": "GB/s", "h2d_bytes_per_step": h2d,
             "d2h_bytes_per_step": d2h, "steps": steps, "ms_per_step": round(ms_step, 3),
-            "host_memory": "pinned" if pinned else "pageable", "per_rank_bytes": True if distributed else None}
+            "host_memory": "pinned" if pinned else "pageable", "per_rank_bytes": True if distributed else None,
+            "path": "C-ABI host entry points (include/lift_host.h)" if not distributed else
+                    "torch H2D copies + shard ops + D2H copy"}
 
 
 def main():

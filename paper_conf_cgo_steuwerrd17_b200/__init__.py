@@ -244,3 +244,47 @@ def lift_sgemv(alpha: float, A: torch.Tensor, x: torch.Tensor, beta: float = 0.0
                            y.data_ptr(), ws.data_ptr() if ws is not None else None, ws.numel() if ws is not None else 0,
                            _stream(dev)))
     return y
+
+
+# ---------------------------------------------------------------------------
+# end to end from host buffers (include/lift_host.h)
+# ---------------------------------------------------------------------------
+def _check_host(t: torch.Tensor, name: str) -> None:
+    if t.dtype != torch.float32 or t.device.type != "cpu" or not t.is_contiguous():
+        raise ValueError(f"{name} must be a contiguous fp32 CPU tensor (pinned for asynchronous copies)")
+
+
+def lift_host_call(op: str, host: dict, dev: dict, alpha: float = 1.0, beta: float = 0.0) -> None:
+    """Enqueue one op from host buffers on the current stream: H2D copies of the
+    inputs into the caller's device buffers, the kernels, the D2H copy of the
+    result (host["out"]).  Synchronise the stream before reading host["out"]."""
+    L = lib()
+    for k, t in host.items():
+        _check_host(t, k)
+    device = next(iter(dev.values())).device
+    s = _stream(device)
+    with torch.cuda.device(device):
+        if op == "dot":
+            n = host["x"].numel()
+            ws = _workspace("dot", device, L.lift_dot_workspace_bytes(n), zero=True)
+            st = L.lift_dot_host(n, host["x"].data_ptr(), host["y"].data_ptr(), host["out"].data_ptr(),
+                                 dev["x"].data_ptr(), dev["y"].data_ptr(), dev["out"].data_ptr(), ws.data_ptr(),
+                                 ws.numel(), s)
+        elif op == "gemv":
+            m, n = host["A"].shape
+            st = L.lift_gemv_host(m, n, host["A"].data_ptr(), host["x"].data_ptr(), host["out"].data_ptr(),
+                                  dev["A"].data_ptr(), dev["x"].data_ptr(), dev["out"].data_ptr(), s)
+        elif op == "gesummv":
+            m, n = host["A"].shape
+            st = L.lift_gesummv_host(m, n, float(alpha), host["A"].data_ptr(), float(beta), host["B"].data_ptr(),
+                                     host["x"].data_ptr(), host["out"].data_ptr(), dev["A"].data_ptr(),
+                                     dev["B"].data_ptr(), dev["x"].data_ptr(), dev["out"].data_ptr(), s)
+        elif op == "atax":
+            m, n = host["A"].shape
+            ws = _workspace("atax", device, L.lift_atax_workspace_bytes(m, n), zero=True)
+            st = L.lift_atax_host(m, n, host["A"].data_ptr(), host["x"].data_ptr(), host["out"].data_ptr(),
+                                  dev["A"].data_ptr(), dev["x"].data_ptr(), dev["out"].data_ptr(), ws.data_ptr(),
+                                  ws.numel(), s)
+        else:
+            raise ValueError(op)
+        check(st)

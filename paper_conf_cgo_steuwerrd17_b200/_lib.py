@@ -54,6 +54,10 @@ SIGNATURES = {
     "lift_gemv_allgather": (i32, [i64, i64, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, u64, vp]),
     "lift_gesummv_allgather": (i32, [i64, i64, f32, vp, f32, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, u64, vp]),
     "lift_atax_reduce": (i32, [i64, i64, vp, vp, vp, vp, sz, vp, i32, i32, i32, u64, i32, vp]),
+    "lift_dot_host": (i32, [i64, vp, vp, vp, vp, vp, vp, vp, sz, vp]),
+    "lift_gemv_host": (i32, [i64, i64, vp, vp, vp, vp, vp, vp, vp]),
+    "lift_gesummv_host": (i32, [i64, i64, f32, vp, f32, vp, vp, vp, vp, vp, vp, vp, vp]),
+    "lift_atax_host": (i32, [i64, i64, vp, vp, vp, vp, vp, vp, vp, sz, vp]),
     "lift_strerror": (ctypes.c_char_p, [i32]),
     "lift_last_cuda_error": (ctypes.c_char_p, []),
     "lift_version": (i32, []),

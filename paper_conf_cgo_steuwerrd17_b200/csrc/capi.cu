@@ -5,11 +5,13 @@
 #include <stdio.h>
 #include <string.h>
 
+#include <initializer_list>
 #include <mutex>
 
 #include "../../include/lift.h"
 #include "../../include/lift_tuning.h"
 #include "../../include/lift_nvlink.h"
+#include "../../include/lift_host.h"
 #include "launch.h"
 
 namespace lift {
@@ -469,6 +471,84 @@ int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float
     return cuda_status(lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream,
                                                make_exch(peers, rank, world, epoch, (int64_t)world * n), dst,
                                                blocks));
+}
+
+// ---------------------------------------------------------------------------
+// end to end from host buffers (lift_host.h)
+// ---------------------------------------------------------------------------
+static int h2d(void *dev, const void *host, uint64_t bytes, lift_stream_t stream) {
+    if (bytes == 0) return LIFT_OK;
+    return cuda_status(cudaMemcpyAsync(dev, host, bytes, cudaMemcpyHostToDevice, (cudaStream_t)stream));
+}
+static int d2h(void *host, const void *dev, uint64_t bytes, lift_stream_t stream) {
+    if (bytes == 0) return LIFT_OK;
+    return cuda_status(cudaMemcpyAsync(host, dev, bytes, cudaMemcpyDeviceToHost, (cudaStream_t)stream));
+}
+static bool any_overlap(std::initializer_list<Range> rs) {
+    const Range *v = rs.begin();
+    const size_t k = rs.size();
+    for (size_t i = 0; i < k; ++i)
+        for (size_t j = i + 1; j < k; ++j)
+            if (overlap(v[i], v[j])) return true;
+    return false;
+}
+
+int lift_dot_host(int64_t n, const float *x_host, const float *y_host, float *result_host, float *x_dev, float *y_dev,
+                  float *result_dev, void *workspace, size_t workspace_bytes, lift_stream_t stream) {
+    if (!size_ok(n, 1)) return LIFT_ERR_BAD_SIZE;
+    if (result_host == nullptr || (n > 0 && (x_host == nullptr || y_host == nullptr))) return LIFT_ERR_NULL_PTR;
+    const uint64_t b = (uint64_t)n * 4;
+    if (x_dev && y_dev && result_dev &&
+        any_overlap({rng(x_dev, b), rng(y_dev, b), rng(result_dev, 4), rng(workspace, workspace_bytes)}))
+        return LIFT_ERR_ALIAS;
+    int st;
+    if ((st = h2d(x_dev, x_host, b, stream)) || (st = h2d(y_dev, y_host, b, stream))) return st;
+    if ((st = lift_dot(n, x_dev, y_dev, result_dev, workspace, workspace_bytes, stream))) return st;
+    return d2h(result_host, result_dev, 4, stream);
+}
+
+int lift_gemv_host(int64_t m, int64_t n, const float *A_host, const float *x_host, float *y_host, float *A_dev,
+                   float *x_dev, float *y_dev, lift_stream_t stream) {
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (m > 0 && (y_host == nullptr || (n > 0 && (A_host == nullptr || x_host == nullptr)))) return LIFT_ERR_NULL_PTR;
+    const uint64_t ba = (uint64_t)m * (uint64_t)n * 4, bx = (uint64_t)n * 4, by = (uint64_t)m * 4;
+    if (any_overlap({rng(A_dev, ba), rng(x_dev, bx), rng(y_dev, by)})) return LIFT_ERR_ALIAS;
+    if (m == 0) return LIFT_OK;
+    int st;
+    if ((st = h2d(A_dev, A_host, ba, stream)) || (st = h2d(x_dev, x_host, bx, stream))) return st;
+    if ((st = lift_gemv(m, n, A_dev, x_dev, y_dev, stream))) return st;
+    return d2h(y_host, y_dev, by, stream);
+}
+
+int lift_gesummv_host(int64_t m, int64_t n, float alpha, const float *A_host, float beta, const float *B_host,
+                      const float *x_host, float *y_host, float *A_dev, float *B_dev, float *x_dev, float *y_dev,
+                      lift_stream_t stream) {
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (m > 0 && (y_host == nullptr || (n > 0 && (A_host == nullptr || B_host == nullptr || x_host == nullptr))))
+        return LIFT_ERR_NULL_PTR;
+    const uint64_t ba = (uint64_t)m * (uint64_t)n * 4, bx = (uint64_t)n * 4, by = (uint64_t)m * 4;
+    if (any_overlap({rng(A_dev, ba), rng(B_dev, ba), rng(x_dev, bx), rng(y_dev, by)})) return LIFT_ERR_ALIAS;
+    if (m == 0) return LIFT_OK;
+    int st;
+    if ((st = h2d(A_dev, A_host, ba, stream)) || (st = h2d(B_dev, B_host, ba, stream)) ||
+        (st = h2d(x_dev, x_host, bx, stream)))
+        return st;
+    if ((st = lift_gesummv(m, n, alpha, A_dev, beta, B_dev, x_dev, y_dev, stream))) return st;
+    return d2h(y_host, y_dev, by, stream);
+}
+
+int lift_atax_host(int64_t m, int64_t n, const float *A_host, const float *x_host, float *y_host, float *A_dev,
+                   float *x_dev, float *y_dev, void *workspace, size_t workspace_bytes, lift_stream_t stream) {
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (n > 0 && (y_host == nullptr || (m > 0 && (A_host == nullptr || x_host == nullptr)))) return LIFT_ERR_NULL_PTR;
+    const uint64_t ba = (uint64_t)m * (uint64_t)n * 4, bx = (uint64_t)n * 4;
+    if (any_overlap({rng(A_dev, ba), rng(x_dev, bx), rng(y_dev, bx), rng(workspace, workspace_bytes)}))
+        return LIFT_ERR_ALIAS;
+    if (n == 0) return LIFT_OK;
+    int st;
+    if ((st = h2d(A_dev, A_host, ba, stream)) || (st = h2d(x_dev, x_host, bx, stream))) return st;
+    if ((st = lift_atax(m, n, A_dev, x_dev, y_dev, workspace, workspace_bytes, stream))) return st;
+    return d2h(y_host, y_dev, bx, stream);
 }
 
 const char *lift_strerror(int status) {

@@ -209,3 +209,12 @@ def test_nvlink_validation():
     wsa = L.lift_atax_workspace_bytes(64, 512)
     assert L.lift_atax_reduce(64, 512, A_, X_, Y_, W_, wsa, peers, 0, 2, 2, 1, 0, None) == SIZE      # dst >= world
     assert L.lift_atax_reduce(64, 510, A_, X_, Y_, W_, wsa, peers, 0, 2, 0, 1, 0, None) == SIZE     # n % 4
+
+
+def test_host_entry_validation():
+    assert L.lift_gemv_host(-1, 4, A_, X_, Y_, A_, X_, Y_, None) == SIZE
+    assert L.lift_gemv_host(4, 4, None, X_, Y_, A_, X_, Y_, None) == NULL
+    assert L.lift_gemv_host(4, 4, A_, X_, Y_, A_, A_ + 8, Y_, None) == ALIAS      # device buffers overlap
+    assert L.lift_gesummv_host(4, 4, 1.0, A_, 1.0, B_, X_, Y_, A_, A_, X_, Y_, None) == ALIAS
+    assert L.lift_dot_host(8, X_, Y_, None, X_, Y_, W_, W_ + 64, 256, None) == NULL
+    assert L.lift_atax_host(0, 0, None, None, None, None, None, None, None, 0, None) == OK

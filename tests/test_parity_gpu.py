@@ -434,3 +434,38 @@ def test_sgemv_alpha1_beta0_is_gemv_bitwise(cuda_device):
     ref = y.clone()
     lift.lift_sgemv(2.0, A, x, -1.0, y)
     assert torch.equal(y, ref)
+
+
+# ===================================================================== host-buffer entry points
+@pytest.mark.parametrize("pinned", [True, False])
+def test_host_entry_points_match_device_path(cuda_device, pinned):
+    m, n = 1000, 4096
+    A = synth.numpy_matrix_rows(synth.SEED_A, n, 0, m)
+    B = synth.numpy_matrix_rows(synth.SEED_B, n, 0, m)
+    x = synth.numpy_uniform(synth.SEED_X, 0, n)
+
+    def host(a):
+        t = torch.from_numpy(np.ascontiguousarray(a))
+        return t.pin_memory() if pinned else t.clone()
+
+    Ad, Bd, xd = dev_np(A, cuda_device), dev_np(B, cuda_device), dev_np(x, cuda_device)
+    cases = {
+        "gemv": (dict(A=host(A), x=host(x), out=host(np.zeros(m, np.float32))),
+                 dict(A=torch.empty_like(Ad), x=torch.empty_like(xd), out=torch.empty(m, device=cuda_device)),
+                 lift.lift_gemv(Ad, xd)),
+        "gesummv": (dict(A=host(A), B=host(B), x=host(x), out=host(np.zeros(m, np.float32))),
+                    dict(A=torch.empty_like(Ad), B=torch.empty_like(Bd), x=torch.empty_like(xd),
+                         out=torch.empty(m, device=cuda_device)),
+                    lift.lift_gesummv(1.5, Ad, 1.2, Bd, xd)),
+        "atax": (dict(A=host(A), x=host(x), out=host(np.zeros(n, np.float32))),
+                 dict(A=torch.empty_like(Ad), x=torch.empty_like(xd), out=torch.empty(n, device=cuda_device)),
+                 lift.lift_atax(Ad, xd)),
+        "dot": (dict(x=host(A.ravel()), y=host(B.ravel()), out=host(np.zeros((), np.float32))),
+                dict(x=torch.empty(m * n, device=cuda_device), y=torch.empty(m * n, device=cuda_device),
+                     out=torch.empty((), device=cuda_device)),
+                lift.lift_dot(Ad.view(-1), Bd.view(-1))),
+    }
+    for op, (h, d, ref) in cases.items():
+        lift.lift_host_call(op, h, d, alpha=1.5, beta=1.2)
+        torch.cuda.synchronize()
+        assert torch.equal(h["out"], ref.cpu()), op
