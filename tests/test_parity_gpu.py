@@ -468,4 +468,4 @@ def test_host_entry_points_match_device_path(cuda_device, pinned):
     for op, (h, d, ref) in cases.items():
         lift.lift_host_call(op, h, d, alpha=1.5, beta=1.2)
         torch.cuda.synchronize()
-        assert torch.equal(h["out"], ref.cpu()), op
+        assert torch.equal(h["out"].reshape(-1), ref.cpu().reshape(-1)), op
