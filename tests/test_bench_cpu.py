@@ -1,0 +1,43 @@
+"""bench.py pieces that need no GPU: the workload matches BASELINE.json, the
+algorithmic byte counts match DESIGN.md §5, and the reference arm (the fp64
+oracle on the host cores) prints a contract line."""
+import json
+import os
+import subprocess
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+import bench  # noqa: E402
+
+
+def test_workload_is_baseline_configs_1_to_4():
+    cfg = json.load(open(os.path.join(ROOT, "BASELINE.json")))["configs"]
+    idx = {w[3] for w in bench.WORKLOAD}
+    assert idx == {1, 2, 3, 4}
+    shapes = {w[0]: w[2] for w in bench.WORKLOAD}
+    assert "4096" in cfg[1] and shapes["gemv_4096x4096"] == dict(m=4096, n=4096)
+    assert "8192" in cfg[2] and shapes["gesummv_8192x8192"] == dict(m=8192, n=8192)
+    assert "8192" in cfg[3] and shapes["atax_8192x8192"] == dict(m=8192, n=8192)
+    assert "65536" in cfg[4] and shapes["gemv_65536x32768"] == dict(m=65536, n=32768)
+    assert "2^31" in cfg[4] and shapes["dot_2^31"] == dict(n=1 << 31)
+
+
+def test_algorithmic_bytes():
+    assert bench.alg_bytes("dot", dict(n=1 << 31)) == 17179869188
+    assert bench.alg_bytes("gemv", dict(m=4096, n=4096)) == 67141632
+    assert bench.alg_bytes("gemv", dict(m=65536, n=32768)) == 8590327808
+    assert bench.alg_bytes("gesummv", dict(m=8192, n=8192)) == 536936448
+    assert bench.alg_bytes("atax", dict(m=8192, n=8192)) == 268500992
+    assert bench.alg_bytes("atax", dict(m=8192, n=8192), "twopass") == 537001984
+
+
+def test_reference_arm_contract_line():
+    r = subprocess.run([sys.executable, "bench.py", "--impl", "reference", "--steps", "1", "--warmup", "1"], cwd=ROOT,
+                       capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0, r.stderr[-2000:]
+    d = json.loads([l for l in r.stdout.splitlines() if l.startswith("{")][-1])
+    assert d["impl"] == "reference" and d["value"] > 0 and d["unit"] == "GB/s"
+    assert d["e2e"]["h2d_bytes_per_step"] == 0 and d["e2e"]["value"] == d["value"]
+    assert d["cpu_baseline"]["kind"] == "oracle" and d["cpu_baseline"]["cores"] >= 1
+    assert d["config"]["workload"] == bench.WORKLOAD_NAME
