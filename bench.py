@@ -609,6 +609,8 @@ def run_e2e(args, bufs, run_op, dev, distributed, world, step_bytes):
             hb["res"].copy_(res.reshape(hb["res"].shape), non_blocking=True)
 
     steps = max(1, min(args.steps, args.e2e_steps))
+    if distributed:  # host buffers take rank-dependent time to pin: align before the first step
+        dist.barrier()
     e2e_step()
     torch.cuda.synchronize()
     if distributed:

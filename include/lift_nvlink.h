@@ -18,7 +18,7 @@
  * order on every rank (the library never resets flags; data is double
  * buffered by epoch parity, so a rank may run at most one call ahead).
  * Every rank must make the matching call, or the waiting ranks trap after
- * ~4 s (cudaErrorLaunchFailure) instead of hanging.
+ * about a minute (cudaErrorLaunchFailure) instead of hanging.
  *
  * Validation follows lift.h (status codes, nothing enqueued on error); the
  * contents of `peers` live in device memory and are not checked.

@@ -52,15 +52,16 @@ __device__ __forceinline__ void exch_signal(const Exch &e, int dst /* -1: all ra
 }
 
 // Wait until every rank has published epoch e.epoch into THIS rank's area.
-// Bounded: a peer that never arrives (a programming error) traps instead of
-// hanging the GPU.
+// Bounded: a peer that never arrives (a programming error) traps after ~1
+// minute instead of hanging the GPU; host-side skew between ranks (allocation,
+// pinning, GC) stays far below that.
 __device__ __forceinline__ void exch_wait_all(const Exch &e) {
     const uint64_t *f = exch_flags(e.peers[e.rank]);
     const long long t0 = clock64();
     for (int r = 0; r < e.world; ++r) {
         while (ld_acquire_sys(f + r) < (uint64_t)e.epoch) {
             __nanosleep(100);
-            if (clock64() - t0 > (1ll << 33)) __trap();  // ~4 s at 2 GHz
+            if (clock64() - t0 > (1ll << 37)) __trap();  // ~70 s at 1.96 GHz
         }
     }
 }
