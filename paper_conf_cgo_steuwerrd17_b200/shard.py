@@ -163,7 +163,7 @@ class FusedGroup:
             if self.transport in ("auto", "symm"):
                 try:
                     ex = ExchangeArea.symmetric(kind, length, self.group)
-                except RuntimeError:
+                except Exception:  # torch symmetric memory unavailable for this group / layout
                     if self.transport == "symm":
                         raise
             if ex is None:  # both transports map the peers' HBM; IPC also works for ranks sharing a GPU
