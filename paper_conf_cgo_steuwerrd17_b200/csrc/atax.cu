@@ -274,6 +274,15 @@ struct FusedPlan {
     size_t smem;  // dynamic smem bytes
 };
 
+// Stage = CR consecutive rows moved by ONE bulk copy; each consumer step takes
+// one stage.  The B200 bulk-copy sweep (tools/readbw.cu bulk,
+// profiles/r01p_readbw_bulk.txt) streams best with copies of >= 32 KiB and about
+// 96-128 KiB in flight per SM (16 KiB copies: 5.2 TB/s; 32 KiB x 3: 7.2 TB/s;
+// 32 KiB x 6: 6.5 TB/s), so CR rows make a ~32 KiB stage (within the register
+// budget of two steps of a[CR][QC]) and the ring holds ~112 KiB.
+constexpr size_t kFusedStageTarget = 32 * 1024;
+constexpr size_t kFusedRingTarget = 112 * 1024;
+
 static bool fused_plan(int64_t n, FusedPlan *p) {
     if (n <= 0 || n % 4 != 0) return false;
     const int64_t nv = n / 4;
@@ -281,24 +290,22 @@ static bool fused_plan(int64_t n, FusedPlan *p) {
     while (qc < 8 && (int64_t)qc * kFusedThreads < nv) qc *= 2;
     if ((int64_t)qc * kFusedThreads < nv) return false;
     const size_t row = (size_t)n * 4;
+    const int cr_max = qc == 1 ? 4 : (qc == 2 ? 2 : 1);  // two steps of a[cr][qc] live in registers
+    int cr = 1;
+    while (cr < cr_max && (size_t)(2 * cr) * row <= kFusedStageTarget) cr *= 2;
+    const size_t stage = (size_t)cr * row;
     const size_t hdr = (size_t)((8 * kFusedMaxStages + 2 * 4 * kFusedWarps * 4) + 127) / 128 * 128;
-    int64_t nst = (int64_t)(((size_t)kFusedSmemBudget - hdr) / row);
+    int64_t nst = (int64_t)((kFusedRingTarget + stage / 2) / stage);
+    if (nst < 2) nst = 2;
     if (nst > kFusedMaxStages) nst = kFusedMaxStages;
-    // rows per step: at most 4 (register budget a[cr][qc]), and small enough
-    // that >= 2 further steps of rows are already in flight (lookahead)
-    int cr = (int)(nst / 3);
-    if (cr > 4) cr = 4;
-    if (qc >= 4 && cr > 2) cr = 2;  // two steps of a[cr][qc] live in registers (software pipeline)
-    if (qc >= 8) cr = 1;
-    if (cr == 3) cr = 2;
-    if (cr < 1) return false;
-    if (nst < cr + 1) return false;
+    while (nst > 2 && hdr + (size_t)nst * stage > (size_t)kFusedSmemBudget) --nst;
+    if (hdr + (size_t)nst * stage > (size_t)kFusedSmemBudget) return false;
     p->qc = qc;
     p->cr = cr;
     p->nst = (int)nst;
     p->hdr = hdr;
     // the drained ring is reused for the final column-sum tile partials
-    const size_t ring = (size_t)nst * row, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
+    const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
     p->smem = hdr + (ring > tile ? ring : tile);
     return true;
 }
@@ -409,7 +416,15 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     const int tid = threadIdx.x;
     const int64_t nv = n / 4;
     const int64_t r0 = m * blockIdx.x / gridDim.x, r1 = m * (blockIdx.x + 1) / gridDim.x;
-    const uint32_t row_bytes = (uint32_t)(n * 4);
+    const size_t stage_floats = (size_t)CR * n;
+    // stage j holds rows [r0 + j*CR, min(r1, r0 + (j+1)*CR)): ONE bulk copy
+    auto issue_stage = [&](int64_t j, int slot) {
+        const int64_t a = r0 + j * CR, b = (a + CR < r1) ? a + CR : r1;
+        const uint32_t bytes = (uint32_t)((b - a) * n * 4);
+        mbar_arrive_expect_tx(full + slot, bytes);
+        bulk_g2s(stage0 + (size_t)slot * stage_floats, A + a * n, bytes, full + slot);
+    };
+    const int64_t nstages = (r1 - r0 + CR - 1) / CR;
 
     if (tid == 0) {
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
@@ -417,10 +432,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     }
     __syncthreads();
     if (tid == 0) {  // prologue: fill the ring
-        for (int i = 0; i < nst && r0 + i < r1; ++i) {
-            mbar_arrive_expect_tx(full + i, row_bytes);
-            bulk_g2s(stage0 + (size_t)i * n, A + (r0 + i) * n, row_bytes, full + i);
-        }
+        for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
     }
 
     float4 xr[QC], yr[QC];
@@ -431,53 +443,38 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         xr[q] = c < nv ? ld_ro4(x4 + c) : zero4();
         yr[q] = zero4();
     }
-    // Software-pipelined over steps: iteration k loads step k's rows and
-    // publishes their partial dots, then applies the rank-1 updates of step
-    // k-1 (whose block reductions are complete).  The one block barrier per
-    // iteration sits at its top, where it also proves that the previous
-    // step's slots have been read into registers, so they are refilled there.
-    int it = 0, buf = 0;   // it = rows loaded so far
-    int prow = 0;          // rows of the previous step (0: none)
-    int64_t prev_r = r0;   // first row of the previous step
-    int slot = 0;          // ring slot of row `it` (it % nst), tracked without division
-    uint32_t phase = 0;    // its mbarrier phase parity ((it / nst) & 1)
-    int pslot = 0;         // ring slot of the previous step's first row
-    float4 ap[CR][QC];     // the previous step's rows, kept for its rank-1 updates
+    // Software-pipelined over steps (one step = one stage of CR rows): iteration
+    // k loads stage k's rows and publishes their partial dots, then applies the
+    // rank-1 updates of stage k-1 (whose block reductions are complete).  The
+    // one block barrier per iteration sits at its top, where it also proves
+    // that stage k-1's slot has been read into registers: thread 0 refills it
+    // there with stage k-1+NST.
+    int buf = 0;
+    int prow = 0;        // rows of the previous stage (0: none)
+    int slot = 0;        // ring slot of stage k (k % nst), tracked without division
+    uint32_t phase = 0;  // its mbarrier phase parity ((k / nst) & 1)
+    int pslot = 0;       // ring slot of stage k-1
+    float4 ap[CR][QC];   // the previous stage's rows, kept for its rank-1 updates
 #pragma unroll
     for (int i = 0; i < CR; ++i)
 #pragma unroll
         for (int q = 0; q < QC; ++q) ap[i][q] = zero4();
-    for (int64_t r = r0;; r += CR, buf ^= 1) {
+    for (int64_t k = 0;; ++k, buf ^= 1) {
+        const int64_t r = r0 + k * CR;
         const int rows = r < r1 ? (int)((r1 - r) < CR ? (r1 - r) : CR) : 0;
-        __syncthreads();  // previous step: partials published, slots consumed
-        if (tid == 0) {
-            for (int i = 0; i < prow; ++i) {
-                const int64_t rn = prev_r + i + nst;  // the row NST ahead reuses this slot
-                if (rn < r1) {
-                    const int st = pslot + i < nst ? pslot + i : pslot + i - nst;
-                    mbar_arrive_expect_tx(full + st, row_bytes);
-                    bulk_g2s(stage0 + (size_t)st * n, A + rn * n, row_bytes, full + st);
-                }
-            }
-        }
+        __syncthreads();  // previous stage: partials published, slot consumed
+        if (tid == 0 && prow > 0 && k - 1 + nst < nstages) issue_stage(k - 1 + nst, pslot);
         float4 a[CR][QC];
         float *rb = red + buf * CR * kFusedWarps;
         if (rows > 0) {
+            mbar_wait_parity(full + slot, phase);
+            const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)slot * stage_floats);
 #pragma unroll
             for (int i = 0; i < CR; ++i) {
-                if (i < rows) {
-                    const bool wrap = slot + i >= nst;
-                    const int st = wrap ? slot + i - nst : slot + i;
-                    mbar_wait_parity(full + st, wrap ? phase ^ 1u : phase);
-                    const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)st * n);
 #pragma unroll
-                    for (int q = 0; q < QC; ++q) {
-                        const int64_t c = tid + (int64_t)kFusedThreads * q;
-                        a[i][q] = c < nv ? S4[c] : zero4();
-                    }
-                } else {
-#pragma unroll
-                    for (int q = 0; q < QC; ++q) a[i][q] = zero4();
+                for (int q = 0; q < QC; ++q) {
+                    const int64_t c = tid + (int64_t)kFusedThreads * q;
+                    a[i][q] = (i < rows && c < nv) ? S4[(int64_t)i * nv + c] : zero4();
                 }
             }
             // partial dots of this thread's columns, CR rows at once
@@ -498,7 +495,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
                 for (int i = 0; i < CR; ++i) rb[i * kFusedWarps + warp] = d[i];
             }
         }
-        // rank-1 updates of the previous step: y += A_r^T t_r
+        // rank-1 updates of the previous stage: y += A_r^T t_r
         if (prow > 0) {
             const float *pb = red + (buf ^ 1) * CR * kFusedWarps;
 #pragma unroll
@@ -526,12 +523,9 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 #pragma unroll
             for (int q = 0; q < QC; ++q) ap[i][q] = a[i][q];
         prow = rows;
-        prev_r = r;
-        it += rows;
         pslot = slot;
-        slot += rows;
-        if (slot >= nst) {
-            slot -= nst;
+        if (++slot == nst) {
+            slot = 0;
             phase ^= 1u;
         }
     }
@@ -615,9 +609,10 @@ static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const flo
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     cudaFuncAttributes a;
     cudaError_t e = cudaFuncGetAttributes(&a, k_atax_fused<1, 4>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<1, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<1, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 2>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<4, 256, 8>);
@@ -646,10 +641,12 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     cudaError_t e = cudaErrorInvalidValue;
 #define LIFT_FUSED_CASE(QC, CR) \
     if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, y, gbar, (int)G, s, ex, dst, cooperative);
+    // fused_plan pairs: qc 1 -> cr 4 (rows <= 8 KiB), qc 2 -> cr 2, qc 4 / 8 -> cr 1
     LIFT_FUSED_CASE(1, 4)
-    LIFT_FUSED_CASE(2, 4)
+    LIFT_FUSED_CASE(1, 2)
+    LIFT_FUSED_CASE(1, 1)
     LIFT_FUSED_CASE(2, 2)
-    LIFT_FUSED_CASE(4, 2)
+    LIFT_FUSED_CASE(2, 1)
     LIFT_FUSED_CASE(4, 1)
     LIFT_FUSED_CASE(8, 1)
 #undef LIFT_FUSED_CASE

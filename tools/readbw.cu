@@ -82,6 +82,52 @@ __global__ void k8(int64_t n8, const float *x, const float *y, float *out) {
     if (s == 12345.f) out[0] = s;
 }
 
+
+// ---- bulk-copy (TMA engine) streaming: one block per SM, ring of NST slots of
+// `chunk` bytes, thread 0 refills a slot as soon as the block has consumed it
+__device__ __forceinline__ uint32_t su32(const void *p) { return (uint32_t)__cvta_generic_to_shared(p); }
+__global__ void __launch_bounds__(256, 1) k_bulk(int64_t bytes_per_block, int chunk, int nst, const char *src,
+                                                 float *out) {
+    extern __shared__ __align__(128) unsigned char sm[];
+    uint64_t *full = (uint64_t *)sm;
+    char *ring = (char *)(sm + 1024);
+    const char *base = src + (int64_t)blockIdx.x * bytes_per_block;
+    const int64_t nchunks = bytes_per_block / chunk;
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < nst; ++i) asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(su32(full + i)));
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncthreads();
+    auto issue = [&](int64_t c) {
+        const int st = (int)(c % nst);
+        asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(su32(full + st)), "r"(chunk)
+                     : "memory");
+        asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                         su32(ring + (int64_t)st * chunk)),
+                     "l"(base + c * chunk), "r"(chunk), "r"(su32(full + st))
+                     : "memory");
+    };
+    if (threadIdx.x == 0)
+        for (int64_t c = 0; c < nst && c < nchunks; ++c) issue(c);
+    float acc = 0.f;
+    for (int64_t c = 0; c < nchunks; ++c) {
+        const int st = (int)(c % nst);
+        const uint32_t ph = (uint32_t)((c / nst) & 1);
+        asm volatile("{\n.reg .pred p;\nW_%=:\nmbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n@!p bra W_%=;\n}\n" ::"r"(
+                         su32(full + st)),
+                     "r"(ph)
+                     : "memory");
+        const float4 *r4 = (const float4 *)(ring + (int64_t)st * chunk);
+        for (int i = threadIdx.x; i < chunk / 16; i += 256) {
+            float4 v = r4[i];
+            acc += v.x + v.y + v.z + v.w;
+        }
+        __syncthreads();
+        if (threadIdx.x == 0 && c + nst < nchunks) issue(c + nst);
+    }
+    if (acc == 12345.f) out[0] = acc;
+}
+
 template <typename K, typename... Args>
 static void run(const char *name, K kern, int tpb, int64_t bytes, Args... args) {
     int per_sm = 0;
@@ -117,6 +163,41 @@ int main(int argc, char **argv) {
     cudaMemset(x, 0, n * 4);
     cudaMemset(y, 0, n * 4);
     const float4 *x4 = (const float4 *)x, *y4 = (const float4 *)y;
+    if (argc > 1 && argv[1][0] == 'b') {
+        // bulk-copy streaming of 256 MiB / 2 GiB: chunk size x ring depth
+        int sms = 0;
+        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
+        for (int64_t total : {(int64_t)256 << 20, (int64_t)2 << 30}) {
+            for (int chunk : {16384, 32768, 65536}) {
+                for (int ring_kb : {96, 192}) {
+                    const int nst = ring_kb * 1024 / chunk;
+                    if (nst < 2) continue;
+                    const int64_t per = total / sms / chunk * chunk;
+                    const size_t smem = 1024 + (size_t)nst * chunk;
+                    cudaFuncSetAttribute(k_bulk, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+                    cudaEvent_t a, b;
+                    cudaEventCreate(&a);
+                    cudaEventCreate(&b);
+                    float best = 1e30f;
+                    for (int it = 0; it < 7; ++it) {
+                        k4<4, 0><<<4 * sms, 256>>>((int64_t)1 << 28, (const float4 *)y, (const float4 *)y, out);
+                        cudaEventRecord(a);
+                        k_bulk<<<sms, 256, smem>>>(per, chunk, nst, (const char *)x, out);
+                        cudaEventRecord(b);
+                        cudaEventSynchronize(b);
+                        float ms;
+                        cudaEventElapsedTime(&ms, a, b);
+                        if (it >= 2 && ms < best) best = ms;
+                    }
+                    printf("bulk %5lld MiB chunk %6d ring %3d KiB (%2d slots)  %9.2f us  %7.1f GB/s\n",
+                           (long long)(total >> 20), chunk, ring_kb, nst, best * 1e3,
+                           (double)per * sms / (best * 1e-3) / 1e9);
+                }
+            }
+        }
+        printf("status %s\n", cudaGetErrorString(cudaGetLastError()));
+        return 0;
+    }
     if (argc > 1) {
         // size sweep: the practical read ceiling of a SINGLE launch of a given size
         // (L2 flushed by reading 1 GiB of y before each timed launch)
