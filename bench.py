@@ -266,15 +266,20 @@ CAPTURE_LABEL = {"gemv_4096x4096": "gemv4096", "gesummv_8192x8192": "gesummv8192
                  "gemv_65536x32768": "gemv65536", "dot_2^31": "dot2p31"}
 
 
-def load_traffic(kernel: str, op_name: str):
-    """ncu --set full DRAM bytes per launch of `kernel` on `op_name`'s shape (profiles/traffic.json)."""
+def load_ncu(kernel: str, op_name: str) -> dict:
+    """The committed ncu --set full capture of `kernel` on `op_name`'s shape (profiles/traffic.json)."""
     p = os.path.join(ROOT, "profiles", "traffic.json")
     try:
         with open(p) as f:
             d = json.load(f)
-        return d.get(f"{kernel}:{CAPTURE_LABEL[op_name]}", {}).get("dram_bytes_per_launch")
+        return d.get(f"{kernel}:{CAPTURE_LABEL[op_name]}", {})
     except Exception:
-        return None
+        return {}
+
+
+def load_traffic(kernel: str, op_name: str):
+    """ncu DRAM bytes (read + write) per launch of `kernel` on `op_name`'s shape."""
+    return load_ncu(kernel, op_name).get("dram_bytes_per_launch")
 
 
 def run_ours(args) -> None:
@@ -483,8 +488,10 @@ def run_ours(args) -> None:
     for i, (name, op, shp, cfg) in enumerate(WORKLOAD):
         by = alg_bytes(op, shp, atax_algo)
         gbs = by / (op_ms[i] * 1e-3) / 1e9
+        kern = {"dot": "k_dot", "gemv": "k_gemv", "gesummv": "k_gemv", "atax": "k_atax_fused"}[op]
         ops[name] = {"configs_index": cfg, "ms": round(op_ms[i], 4), "alg_bytes": by, "GB_s": round(gbs, 1),
-                     "frac_of_peak_per_gpu": round(gbs / world / peak, 4)}
+                     "frac_of_peak_per_gpu": round(gbs / world / peak, 4),
+                     "ncu_dram_pct_of_peak": load_ncu(kern, name).get("ncu_dram_pct_of_peak")}
     dom_name, dom_op, dom_shp, _ = WORKLOAD[dom]
     kernel = {"dot": "k_dot", "gemv": "k_gemv", "gesummv": "k_gemv", "atax": "k_atax_fused"}[dom_op]
     dom_bytes_rank = alg_bytes(dom_op, dom_shp, atax_algo) / world  # per launch, per rank
@@ -513,7 +520,9 @@ def run_ours(args) -> None:
     achieved = dom_bytes_rank / (kms * 1e-3) / 1e9
     roofline = {"bound": "hbm", "kernel": kernel, "op": dom_name, "achieved": round(achieved, 1), "peak": peak,
                 "unit": "GB/s", "frac": round(achieved / peak, 4), "traffic": load_traffic(kernel, dom_name),
-                "alg_bytes_per_launch": int(dom_bytes_rank), "launch_ms": round(kms, 4), "peak_source": peak_src}
+                "alg_bytes_per_launch": int(dom_bytes_rank), "launch_ms": round(kms, 4), "peak_source": peak_src,
+                "ncu_dram_pct_of_peak": load_ncu(kernel, dom_name).get("ncu_dram_pct_of_peak"),
+                "ncu_source": load_ncu(kernel, dom_name).get("source")}
 
     kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 1}[op] for _, op, _, _ in WORKLOAD)
     gpu_launches = kernels_per_step * args.steps

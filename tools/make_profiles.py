@@ -117,8 +117,15 @@ def main(tag, prefix):
                 b = num(vals["dram__bytes_read.sum"]) * unit.get(vals["dram__bytes_read.sum"][0], 1) + \
                     num(vals["dram__bytes_write.sum"]) * unit.get(vals["dram__bytes_write.sum"][0], 1)
                 kern = name.split("(")[0].replace("void ", "").split("<")[0].strip()
-                traffic[kern + ":" + label] = {"dram_bytes_per_launch": b,
-                                               "source": f"profiles/{prefix}_ncu_full_{label}.txt"}
+                ent = {"dram_bytes_per_launch": b, "source": f"profiles/{prefix}_ncu_full_{label}.txt"}
+                pct = vals.get("gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed")
+                if pct is not None:
+                    ent["ncu_dram_pct_of_peak"] = round(float(pct[1].replace(",", "")), 2)
+                dur = vals.get("gpu__time_duration.sum")
+                if dur is not None:
+                    scale = {"ns": 1e-3, "usecond": 1.0, "us": 1.0, "ms": 1e3, "msecond": 1e3}.get(dur[0], 1.0)
+                    ent["ncu_duration_us"] = round(float(dur[1].replace(",", "")) * scale, 3)
+                traffic[kern + ":" + label] = ent
     json.dump(traffic, open(tj, "w"), indent=1, sort_keys=True)
 
 
