@@ -128,6 +128,17 @@ __global__ void __launch_bounds__(256, 1) k_bulk(int64_t bytes_per_block, int ch
     if (acc == 12345.f) out[0] = acc;
 }
 
+// fill with non-constant data (zero pages may be served compressed)
+__global__ void k_fill(float *p, int64_t n, uint32_t seed) {
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (int64_t)gridDim.x * blockDim.x) {
+        uint32_t h = (uint32_t)i * 2654435761u ^ seed;
+        h ^= h >> 16;
+        h *= 0x7feb352du;
+        h ^= h >> 15;
+        p[i] = (float)(h >> 8) * (1.0f / 16777216.0f) - 0.5f;
+    }
+}
+
 template <typename K, typename... Args>
 static void run(const char *name, K kern, int tpb, int64_t bytes, Args... args) {
     int per_sm = 0;
@@ -160,8 +171,9 @@ int main(int argc, char **argv) {
     cudaMalloc(&x, n * 4);
     cudaMalloc(&y, n * 4);
     cudaMalloc(&out, 64);
-    cudaMemset(x, 0, n * 4);
-    cudaMemset(y, 0, n * 4);
+    k_fill<<<4096, 256>>>(x, n, 1u);
+    k_fill<<<4096, 256>>>(y, n, 2u);
+    cudaDeviceSynchronize();
     const float4 *x4 = (const float4 *)x, *y4 = (const float4 *)y;
     if (argc > 1 && argv[1][0] == 'b') {
         // bulk-copy streaming of 256 MiB / 2 GiB: chunk size x ring depth
