@@ -16,6 +16,23 @@
  *           batches in flight); 0 = automatic
  * The scalar path (n % 4 != 0 or a base not 16-byte aligned) has one shape:
  * wpr = 1, rg = 8, lb = 4 (or 0 for each).
+ *
+ * lift_atax_fused_tuned: lift_atax with the single-pass fused kernel
+ * (lift_atax_algo_run(LIFT_ATAX_FUSED, ...): same arguments, workspace and
+ * validation; for any nst / l2_ahead the results are bitwise identical to it —
+ * the summation order depends only on (m, n), the SM count and the row
+ * assignment):
+ *   nst       stages (one bulk copy of ~32 KiB of rows each) in the shared-
+ *             memory ring, 2..16 and within the shared-memory budget
+ *             (0 = automatic)
+ *   l2_ahead  stages prefetched into L2 (cp.async.bulk.prefetch) beyond the
+ *             ring, 0..64 (-1 = automatic)
+ *   cyclic    1 = block b streams row stages b, b+G, b+2G, ... (G blocks),
+ *             0 = block b streams one contiguous band of rows (-1 = automatic);
+ *             this changes which rows each block's partial sums, so results
+ *             are bitwise those of the untuned call only at the automatic
+ *             setting
+ *
  * An unsupported combination returns LIFT_ERR_CUDA with
  * lift_last_cuda_error() = "invalid argument".
  */
@@ -34,6 +51,10 @@ LIFT_API int lift_gemv_tuned(int64_t m, int64_t n, const float *A, const float *
 LIFT_API int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *A, float beta,
                        const float *B, const float *x, float *y,
                        int wpr, int rg, int blocks, int xsmem, int lb, lift_stream_t stream);
+
+LIFT_API int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y,
+                                   void *workspace, size_t workspace_bytes, int nst, int l2_ahead, int cyclic,
+                                   lift_stream_t stream);
 
 #ifdef __cplusplus
 }

@@ -19,6 +19,7 @@ from ._lib import (LIFT_ATAX_AUTO, LIFT_ATAX_FUSED, LIFT_ATAX_TWOPASS, LiftError
                    check, lib, library_path)
 
 __all__ = ["lift_dot", "lift_gemv", "lift_gesummv", "lift_atax", "lift_gemv_tuned", "lift_gesummv_tuned",
+           "lift_atax_fused_tuned",
            "lift_partial_dot", "lift_dot_listing1", "lift_sgemv",
            "LiftError", "lib", "library_path", "KERNELS_PER_CALL"]
 
@@ -172,6 +173,27 @@ def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None,
         ws = _workspace("atax", dev, nbytes, zero=True)
         check(L.lift_atax_algo_run(_ALGOS[algo], m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(),
                                    ws.numel(), _stream(dev)))
+    return out
+
+
+def lift_atax_fused_tuned(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None, nst: int = 0,
+                          l2_ahead: int = -1, cyclic: int = -1) -> torch.Tensor:
+    """lift_atax(algo="fused") with the ring depth / L2 prefetch distance overridden (lift_tuning.h)."""
+    _check_tensor(A, "A", 2)
+    _check_tensor(x, "x", 1)
+    dev = _same_device(A, x)
+    m, n = A.shape
+    if x.numel() != n:
+        raise ValueError(f"x has {x.numel()} elements, A has {n} columns")
+    if out is None:
+        out = torch.empty(n, dtype=torch.float32, device=dev)
+    _check_tensor(out, "out", 1)
+    L = lib()
+    nbytes = L.lift_atax_workspace_bytes(m, n)
+    with torch.cuda.device(dev):
+        ws = _workspace("atax", dev, nbytes, zero=True)
+        check(L.lift_atax_fused_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
+                                      nst, l2_ahead, cyclic, _stream(dev)))
     return out
 
 

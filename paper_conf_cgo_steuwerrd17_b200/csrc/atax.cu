@@ -15,12 +15,13 @@
 //   3. k_colsum         y_j = sum_s partials[s][j] in a fixed order
 //
 // FUSED (single pass, reads A once): persistent blocks, one per SM, each owning
-// a contiguous band of rows.  A producer warp streams rows of A into a ring of
-// shared-memory stages with the bulk-copy engine (cp.async.bulk + mbarrier
-// full/empty pairs, SASS UBLKCP).  512 consumer threads each own fixed vector
-// columns with x for those columns in registers; per row they compute the
-// partial dot, reduce it across the block (warp butterfly + one named barrier)
-// to t_r = A_r . x, and fold A_rj * t_r into their y registers from the SAME
+// a contiguous band of rows.  Thread 0 streams stages of CR rows (~32 KiB) of
+// A into a ring of shared-memory slots with the bulk-copy engine (one
+// cp.async.bulk + one "full" mbarrier per slot, SASS UBLKCP).  512 threads
+// each own fixed vector columns with x for those columns in registers; per
+// stage they compute the partial dots, reduce them across the block (warp
+// butterfly + smem, one block barrier per software-pipelined step) to
+// t_r = A_r . x, and fold A_rj * t_r into their y registers from the SAME
 // registers — t is never written, A is read once (4*m*n bytes instead of 8).
 // The per-block y partials are summed in a fixed order in the SAME launch: a
 // grid barrier (cooperative launch, one block per SM) and then every block
@@ -65,23 +66,21 @@ __device__ __forceinline__ void colsum_tile(int S, int64_t nv, const float *__re
 #pragma unroll
     for (int e = 0; e < VEC; ++e) acc[e] = 0.f;
     if (c < nv) {
-        int s = s0;
-        for (; s + 4 <= s1; s += 4) {
-            V v[4];
+        // in order, 8 predicated loads in flight (a ragged chunk costs one L2
+        // latency, not one per leftover row)
+        for (int s = s0; s < s1; s += 8) {
+            V v[8];
 #pragma unroll
-            for (int u = 0; u < 4; ++u) v[u] = __ldcg(PV + (int64_t)(s + u) * nv + c);
+            for (int u = 0; u < 8; ++u)
+                if (s + u < s1) v[u] = __ldcg(PV + (int64_t)(s + u) * nv + c);
 #pragma unroll
-            for (int u = 0; u < 4; ++u) {
-                const float *f = reinterpret_cast<const float *>(&v[u]);
+            for (int u = 0; u < 8; ++u) {
+                if (s + u < s1) {
+                    const float *f = reinterpret_cast<const float *>(&v[u]);
 #pragma unroll
-                for (int e = 0; e < VEC; ++e) acc[e] = __fadd_rn(acc[e], f[e]);
+                    for (int e = 0; e < VEC; ++e) acc[e] = __fadd_rn(acc[e], f[e]);
+                }
             }
-        }
-        for (; s < s1; ++s) {
-            V v = __ldcg(PV + (int64_t)s * nv + c);
-            const float *f = reinterpret_cast<const float *>(&v);
-#pragma unroll
-            for (int e = 0; e < VEC; ++e) acc[e] = __fadd_rn(acc[e], f[e]);
         }
     }
 #pragma unroll
@@ -270,6 +269,8 @@ struct FusedPlan {
     int qc;       // float4 columns per thread (1, 2, 4, 8)
     int cr;       // rows per step
     int nst;      // stages (rows) in the ring
+    int l2a;      // stages prefetched into L2 beyond the ring
+    int cyc;      // 1: stages assigned to blocks cyclically, 0: contiguous bands
     size_t hdr;   // barrier + reduction header bytes
     size_t smem;  // dynamic smem bytes
 };
@@ -282,8 +283,10 @@ struct FusedPlan {
 // budget of two steps of a[CR][QC]) and the ring holds ~112 KiB.
 constexpr size_t kFusedStageTarget = 32 * 1024;
 constexpr size_t kFusedRingTarget = 112 * 1024;
+constexpr int kFusedL2Ahead = 0;
+constexpr int kFusedCyclic = 1;
 
-static bool fused_plan(int64_t n, FusedPlan *p) {
+static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}) {
     if (n <= 0 || n % 4 != 0) return false;
     const int64_t nv = n / 4;
     int qc = 1;
@@ -299,10 +302,17 @@ static bool fused_plan(int64_t n, FusedPlan *p) {
     if (nst < 2) nst = 2;
     if (nst > kFusedMaxStages) nst = kFusedMaxStages;
     while (nst > 2 && hdr + (size_t)nst * stage > (size_t)kFusedSmemBudget) --nst;
+    if (tune.nst != 0) {  // explicit ring depth (lift_tuning.h): must fit as given
+        if (tune.nst < 2 || tune.nst > kFusedMaxStages) return false;
+        nst = tune.nst;
+    }
     if (hdr + (size_t)nst * stage > (size_t)kFusedSmemBudget) return false;
+    if (tune.l2a < -1 || tune.l2a > 64 || tune.cyc < -1 || tune.cyc > 1) return false;
     p->qc = qc;
     p->cr = cr;
     p->nst = (int)nst;
+    p->l2a = tune.l2a >= 0 ? tune.l2a : kFusedL2Ahead;
+    p->cyc = tune.cyc >= 0 ? tune.cyc : kFusedCyclic;
     p->hdr = hdr;
     // the drained ring is reused for the final column-sum tile partials
     const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
@@ -324,6 +334,7 @@ bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
 // (each thread folds ~S/32 rows in order, all loads in flight), then the 32
 // split sums of a column are combined by a pairwise tree.  Deterministic:
 // the order depends only on S.
+template <int IF /* loads in flight per thread */>
 __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__restrict__ P, float *__restrict__ y,
                                              int64_t c0, int64_t c1, float4 *part /* smem [32][16] */) {
     constexpr int CW = 16, SPL = 32;
@@ -335,25 +346,22 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
         const int64_t c = cb + col;
         float4 acc = zero4();
         if (c < c1) {
-            int s = s0;
-            for (; s + 8 <= s1; s += 8) {
-                float4 v[8];
+            // in order, IF predicated loads in flight (S/32 is ~5 rows here: one
+            // or two L2 latencies instead of five)
+            for (int s = s0; s < s1; s += IF) {
+                float4 v[IF];
 #pragma unroll
-                for (int u = 0; u < 8; ++u) v[u] = __ldcg(P4 + (int64_t)(s + u) * nv + c);
+                for (int u = 0; u < IF; ++u)
+                    if (s + u < s1) v[u] = __ldcg(P4 + (int64_t)(s + u) * nv + c);
 #pragma unroll
-                for (int u = 0; u < 8; ++u) {
-                    acc.x = __fadd_rn(acc.x, v[u].x);
-                    acc.y = __fadd_rn(acc.y, v[u].y);
-                    acc.z = __fadd_rn(acc.z, v[u].z);
-                    acc.w = __fadd_rn(acc.w, v[u].w);
+                for (int u = 0; u < IF; ++u) {
+                    if (s + u < s1) {
+                        acc.x = __fadd_rn(acc.x, v[u].x);
+                        acc.y = __fadd_rn(acc.y, v[u].y);
+                        acc.z = __fadd_rn(acc.z, v[u].z);
+                        acc.w = __fadd_rn(acc.w, v[u].w);
+                    }
                 }
-            }
-            for (; s < s1; ++s) {
-                const float4 v = __ldcg(P4 + (int64_t)s * nv + c);
-                acc.x = __fadd_rn(acc.x, v.x);
-                acc.y = __fadd_rn(acc.y, v.y);
-                acc.z = __fadd_rn(acc.z, v.z);
-                acc.w = __fadd_rn(acc.w, v.w);
             }
         }
         part[sp * CW + col] = acc;
@@ -406,7 +414,7 @@ template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
     k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
                  float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar, Exch ex,
-                 int dst) {
+                 int dst, int l2a, int cyc) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
@@ -415,24 +423,41 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int tid = threadIdx.x;
     const int64_t nv = n / 4;
-    const int64_t r0 = m * blockIdx.x / gridDim.x, r1 = m * (blockIdx.x + 1) / gridDim.x;
     const size_t stage_floats = (size_t)CR * n;
-    // stage j holds rows [r0 + j*CR, min(r1, r0 + (j+1)*CR)): ONE bulk copy
-    auto issue_stage = [&](int64_t j, int slot) {
-        const int64_t a = r0 + j * CR, b = (a + CR < r1) ? a + CR : r1;
-        const uint32_t bytes = (uint32_t)((b - a) * n * 4);
-        mbar_arrive_expect_tx(full + slot, bytes);
-        bulk_g2s(stage0 + (size_t)slot * stage_floats, A + a * n, bytes, full + slot);
+    // This block's stages (CR consecutive rows each, ONE bulk copy): either a
+    // contiguous band of rows [r0, r1) (cyc = 0), or every G-th stage of the
+    // whole matrix (cyc = 1: at any moment all blocks read one ~G*CR-row
+    // window of A).  The assignment is fixed by (m, n, G): deterministic.
+    const int64_t G = gridDim.x, bid = blockIdx.x;
+    const int64_t r0 = cyc ? 0 : m * bid / G, r1 = cyc ? m : m * (bid + 1) / G;
+    const int64_t all_stages = (m + CR - 1) / CR;
+    const int64_t nstages = cyc ? (bid < all_stages ? (all_stages - bid + G - 1) / G : 0) : (r1 - r0 + CR - 1) / CR;
+    auto stage_row = [&](int64_t j) -> int64_t { return cyc ? (j * G + bid) * CR : r0 + j * CR; };
+    auto stage_rows = [&](int64_t j) -> int {
+        if (j >= nstages) return 0;
+        const int64_t a = stage_row(j);
+        return (int)((r1 - a) < CR ? (r1 - a) : CR);
     };
-    const int64_t nstages = (r1 - r0 + CR - 1) / CR;
+    auto issue_stage = [&](int64_t j, int slot) {
+        const uint32_t bytes = (uint32_t)((int64_t)stage_rows(j) * n * 4);
+        mbar_arrive_expect_tx(full + slot, bytes);
+        bulk_g2s(stage0 + (size_t)slot * stage_floats, A + stage_row(j) * n, bytes, full + slot);
+    };
+    // optional deeper pipeline without smem: stage j is prefetched into L2 when
+    // stage j - l2a enters the ring
+    auto prefetch_stage = [&](int64_t j) {
+        if (j >= nstages) return;
+        bulk_prefetch_l2(A + stage_row(j) * n, (uint32_t)((int64_t)stage_rows(j) * n * 4));
+    };
 
     if (tid == 0) {
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         fence_mbar_init();
     }
     __syncthreads();
-    if (tid == 0) {  // prologue: fill the ring
+    if (tid == 0) {  // prologue: fill the ring (and the L2 prefetch window beyond it)
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
+        for (int i = 0; i < l2a; ++i) prefetch_stage(nst + i);
     }
 
     float4 xr[QC], yr[QC];
@@ -460,10 +485,12 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 #pragma unroll
         for (int q = 0; q < QC; ++q) ap[i][q] = zero4();
     for (int64_t k = 0;; ++k, buf ^= 1) {
-        const int64_t r = r0 + k * CR;
-        const int rows = r < r1 ? (int)((r1 - r) < CR ? (r1 - r) : CR) : 0;
+        const int rows = stage_rows(k);
         __syncthreads();  // previous stage: partials published, slot consumed
-        if (tid == 0 && prow > 0 && k - 1 + nst < nstages) issue_stage(k - 1 + nst, pslot);
+        if (tid == 0 && prow > 0 && k - 1 + nst < nstages) {
+            issue_stage(k - 1 + nst, pslot);
+            if (l2a > 0) prefetch_stage(k - 1 + nst + l2a);
+        }
         float4 a[CR][QC];
         float *rb = red + buf * CR * kFusedWarps;
         if (rows > 0) {
@@ -541,7 +568,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     grid_barrier(gbar);
     // every block sums its own slice of columns (the drained ring holds the split sums)
     const int64_t c0 = nv * blockIdx.x / gridDim.x, c1 = nv * (blockIdx.x + 1) / gridDim.x;
-    colsum_slice((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0));
+    colsum_slice<8>((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0));
     if (ex.world == 0) {
         grid_depart(gbar);
         return;
@@ -603,7 +630,7 @@ static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const flo
     attr[0].val.cooperative = 1;
     cfg.attrs = attr;
     cfg.numAttrs = cooperative ? 1 : 0;
-    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst);
+    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.l2a, p.cyc);
 }
 
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)
@@ -623,11 +650,11 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
 }
 
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
-                              void *ws, cudaStream_t s, Exch ex, int dst, int blocks) {
+                              void *ws, cudaStream_t s, Exch ex, int dst, int blocks, FusedTuning tune) {
     if (n == 0) return cudaSuccess;
-    if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
     FusedPlan p;
-    if (!fused_plan(n, &p)) return cudaErrorInvalidValue;
+    if (!fused_plan(n, &p, tune)) return cudaErrorInvalidValue;
+    if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
     unsigned int *gbar = static_cast<unsigned int *>(ws);
     float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
     int64_t G = d.sms;

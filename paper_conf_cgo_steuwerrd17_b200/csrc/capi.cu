@@ -231,6 +231,37 @@ int lift_atax(int64_t m, int64_t n, const float *A, const float *x, float *y, vo
     return lift_atax_algo_run(LIFT_ATAX_AUTO, m, n, A, x, y, workspace, workspace_bytes, stream);
 }
 
+int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
+                          size_t workspace_bytes, int nst, int l2_ahead, int cyclic, lift_stream_t stream) {
+    // validation of lift_atax_algo_run(LIFT_ATAX_FUSED, ...), then the overrides
+    if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (n > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
+    if (m > 0 && n > 0 && (A == nullptr || x == nullptr)) return LIFT_ERR_NULL_PTR;
+    if (n > 0 && mis4(y)) return LIFT_ERR_MISALIGNED;
+    if (m > 0 && n > 0 && (mis4(A) || mis4(x))) return LIFT_ERR_MISALIGNED;
+    if (workspace == nullptr || workspace_bytes < lift_atax_workspace_bytes(m, n) ||
+        (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
+        return LIFT_ERR_WORKSPACE;
+    const uint64_t mat = (uint64_t)m * (uint64_t)n * 4;
+    const Range ry = rng(y, (uint64_t)n * 4), rw = rng(workspace, workspace_bytes);
+    const Range rA = rng(A, mat), rx = rng(x, (uint64_t)n * 4);
+    if (overlap(ry, rA) || overlap(ry, rx) || overlap(ry, rw) || overlap(rw, rA) || overlap(rw, rx))
+        return LIFT_ERR_ALIAS;
+    const bool aligned = ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
+                           reinterpret_cast<uintptr_t>(y)) & 15) == 0;
+    if (m > 0 && n > 0 && !lift::atax_fused_supported(m, n, aligned)) return LIFT_ERR_BAD_SIZE;
+    if (n == 0) return LIFT_OK;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    lift::FusedTuning t;
+    t.nst = nst;
+    t.l2a = l2_ahead;
+    t.cyc = cyclic;
+    return cuda_status(
+        lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream, lift::Exch{}, -1, 0, t));
+}
+
 // (layout, trans) -> does the row-major kernel walk rows of the stored matrix (false)
 // or its columns (true)?  Column-major A is the row-major A^T.
 static bool sgemv_colpath(int layout, int trans) { return (layout == 0) == (trans == 1); }

@@ -129,6 +129,12 @@ __device__ __forceinline__ void bulk_g2s(void *dst_smem, const void *src_gmem, u
         : "memory");
 }
 
+// Prefetch `bytes` (multiple of 16) of gmem into L2 with the bulk-copy engine
+// (no smem, no completion tracking).
+__device__ __forceinline__ void bulk_prefetch_l2(const void *src_gmem, uint32_t bytes) {
+    asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(src_gmem), "r"(bytes) : "memory");
+}
+
 // Stage `bytes` (multiple of 16) of gmem into smem with the bulk-copy engine.
 // Called by ALL threads of the block; thread 0 issues. Returns after the data
 // has landed (mbarrier phase 0 completes).  `bar` must be a fresh mbarrier

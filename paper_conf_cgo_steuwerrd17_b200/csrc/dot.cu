@@ -102,9 +102,18 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
     __syncthreads();
     if (!am_last) return;
     // second stage (L422-426), fixed order: thread j folds partials j, j+TPB, ...
+    // (8 predicated loads in flight, added in that order)
     __threadfence();
     float p = 0.f;
-    for (int j = threadIdx.x; j < (int)gridDim.x; j += TPB) p = __fadd_rn(p, __ldcg(partials + j));
+    for (int j0 = threadIdx.x; j0 < (int)gridDim.x; j0 += 8 * TPB) {
+        float v[8];
+#pragma unroll
+        for (int u = 0; u < 8; ++u)
+            if (j0 + u * TPB < (int)gridDim.x) v[u] = __ldcg(partials + j0 + u * TPB);
+#pragma unroll
+        for (int u = 0; u < 8; ++u)
+            if (j0 + u * TPB < (int)gridDim.x) p = __fadd_rn(p, v[u]);
+    }
     __syncthreads();  // red[] reuse
     float tot = block_sum<TPB, U>(p, red);
     if (threadIdx.x == 0) {

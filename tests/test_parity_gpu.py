@@ -286,6 +286,36 @@ def test_atax_parity(cuda_device, m, n, algo):
     assert_tol(got, ref, mag, f"atax {m}x{n} {algo}")
 
 
+def test_atax_fused_tuning(cuda_device):
+    """lift_atax_fused_tuned: the ring depth and the L2 prefetch distance
+    change only the speed (bitwise equal results); the row assignment
+    (banded / cyclic) changes which rows each block's partial sums, so both
+    are checked against the oracle, and the automatic setting is one of them
+    bitwise; unsupported settings are rejected."""
+    for m, n in ((1000, 4096), (777, 8192), (300, 16384), (5000, 512)):
+        A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+        x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+        ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+        auto = lift.lift_atax(A, x, algo="fused")
+        hits = 0
+        for cyc in (0, 1):
+            base = lift.lift_atax_fused_tuned(A, x, cyclic=cyc)
+            assert_tol(base.cpu().numpy(), ref, mag, f"atax tuned {m}x{n} cyc {cyc}")
+            hits += int(torch.equal(base, auto))
+            for nst in (2, 3, 5):
+                for l2a in (0, 1, 3):
+                    try:
+                        got = lift.lift_atax_fused_tuned(A, x, nst=nst, l2_ahead=l2a, cyclic=cyc)
+                    except lift.LiftError:  # ring does not fit the shared-memory budget
+                        assert n >= 8192 and nst >= 5, (m, n, nst)
+                        continue
+                    assert torch.equal(got, base), (m, n, cyc, nst, l2a)
+        assert hits >= 1
+        for bad in (dict(nst=1), dict(nst=17), dict(l2_ahead=65), dict(cyclic=2)):
+            with pytest.raises(lift.LiftError):
+                lift.lift_atax_fused_tuned(A, x, **bad)
+
+
 @pytest.mark.parametrize("algo", ["fused", "twopass"])
 def test_atax_full_size_8192(cuda_device, algo):
     """configs[3] at one GPU, every output."""

@@ -214,7 +214,8 @@ int main(int argc, char **argv) {
         // size sweep: the practical read ceiling of a SINGLE launch of a given size
         // (L2 flushed by reading 1 GiB of y before each timed launch)
         for (int64_t bytes : {(int64_t)8 << 20, (int64_t)64 << 20, (int64_t)256 << 20, (int64_t)512 << 20,
-                              (int64_t)2 << 30, (int64_t)8 << 30}) {
+                              (int64_t)2 << 30, (int64_t)4 << 30}) {
+            // two arrays of bytes/8 floats each, both inside x (4 GiB)
             const int64_t m = bytes / 8;  // elements per array
             int sms = 0, per_sm = 0;
             cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
