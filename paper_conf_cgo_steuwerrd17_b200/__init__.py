@@ -55,13 +55,26 @@ def _stream(device: torch.device) -> int:
     return torch.cuda.current_stream(device).cuda_stream
 
 
+def _capture_id(stream: int) -> int:
+    """Id of the CUDA-graph capture sequence `stream` is in (unique per process)."""
+    from cuda.bindings import runtime as rt
+    err, _status, cid = rt.cudaStreamGetCaptureInfo(stream)[:3]
+    if int(err) != 0:
+        raise RuntimeError(f"cudaStreamGetCaptureInfo failed: {err}")
+    return int(cid)
+
+
 def _workspace(kind: str, device: torch.device, nbytes: int, zero: bool) -> torch.Tensor:
-    """Per-(kind, device, stream) cached workspace, grown on demand.
+    """Per-(kind, device, stream, capture) cached workspace, grown on demand.
 
     The dot and ATAX workspaces start with counters that must be zero before
     first use; they are allocated with torch.zeros and every call leaves them
-    zero again."""
-    key = (kind, device.index, _stream(device))
+    zero again.  A workspace first allocated while a CUDA graph is being
+    captured is zeroed only when that graph replays, so it is keyed by the
+    capture sequence and never handed to eager calls or to another graph."""
+    stream = _stream(device)
+    cid = _capture_id(stream) if torch.cuda.is_current_stream_capturing() else 0
+    key = (kind, device.index, stream, cid)
     with _ws_lock:
         ws = _ws_cache.get(key)
         if ws is None or ws.numel() < nbytes:

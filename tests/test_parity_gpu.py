@@ -209,6 +209,40 @@ def test_gemv_nondefault_stream_and_graph(cuda_device):
     assert torch.equal(y2, ref)
 
 
+def test_workspace_per_graph_capture(cuda_device):
+    """Workspaces with counters (dot ticket, ATAX grid barrier) first made
+    inside a graph capture are zeroed only when that graph replays: each
+    capture gets its own, and each graph alone replays correctly."""
+    from paper_conf_cgo_steuwerrd17_b200 import _ws_cache
+    n = 1 << 20
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    y = synth.torch_uniform(synth.SEED_Y, 0, n, device=cuda_device)
+    A = synth.torch_matrix_rows(synth.SEED_A, 1024, 0, 700, device=cuda_device)
+    xa = synth.torch_uniform(synth.SEED_X, 0, 1024, device=cuda_device)
+    want_d, want_a = lift.lift_dot(x, y).clone(), lift.lift_atax(A, xa).clone()
+    before = {k for k in _ws_cache if k[3] != 0}
+    graphs, outs = [], []
+    for _ in range(2):
+        g = torch.cuda.CUDAGraph()
+        d = torch.empty((), device=cuda_device)
+        a = torch.empty(1024, device=cuda_device)
+        with torch.cuda.graph(g):
+            lift.lift_dot(x, y, out=d)
+            lift.lift_atax(A, xa, out=a)
+        graphs.append(g)
+        outs.append((d, a))
+    new = {k for k in _ws_cache if k[3] != 0} - before
+    assert len({k[3] for k in new}) == 2 and {k[0] for k in new} == {"dot", "atax"}
+    for g, (d, a) in reversed(list(zip(graphs, outs))):  # the second graph first, alone
+        d.zero_()
+        a.zero_()
+        for _ in range(3):
+            g.replay()
+        torch.cuda.synchronize()
+        assert torch.equal(d, want_d) and torch.equal(a, want_a)
+    assert torch.equal(lift.lift_dot(x, y), want_d)  # the eager workspace is untouched
+
+
 @pytest.mark.slow
 def test_gemv_full_size_65536x32768_sampled(cuda_device):
     """configs[4] large GEMV (8 GiB A) in the bench's launch configuration;
