@@ -41,3 +41,10 @@ def test_reference_arm_contract_line():
     assert d["e2e"]["h2d_bytes_per_step"] == 0 and d["e2e"]["value"] == d["value"]
     assert d["cpu_baseline"]["kind"] == "oracle" and d["cpu_baseline"]["cores"] >= 1
     assert d["config"]["workload"] == bench.WORKLOAD_NAME
+
+
+def test_peaks():
+    # measured copy peak from the driver's file; theoretical HBM3e peak from its memory clock
+    peak, src = bench.measured_peak()
+    assert peak > 1000 and src
+    assert abs(bench.spec_peak() - 3996e6 * 2 * 8192 / 8 / 1e9) < 50
