@@ -26,6 +26,10 @@ sides of exactly K timed steps; device time from CUDA events on the launching
 stream; max over ranks; SM clocks + throttle reasons sampled through NVML
 during the timed region.
 
+N > 1 (torchrun, one rank per GPU): each op's one collective is fused into
+its kernel over NVLink peer memory (include/lift_nvlink.h) after a self-check
+against the torch.distributed/NCCL path, else NCCL (--collectives).
+
 `--impl reference` times the fp64 CPU oracle (oracle/, the reference arm of
 this tier) on a bounded sample of the same workload on the host cores.
 """
@@ -342,8 +346,21 @@ def run_ours(args) -> None:
         bufs[name] = b
     torch.cuda.synchronize()
 
-    fused = distributed and args.collectives == "fused"
+    # N > 1: the collective fused into the kernels (NEXT-2) unless --collectives nccl;
+    # "auto" first checks the fused ops against the NCCL ones on a small problem
+    # and falls back to NCCL (saying why) if any rank fails
+    fused = distributed and args.collectives in ("auto", "fused")
     fg = shard.FusedGroup() if fused else None
+    collectives = None
+    if distributed:
+        collectives = "fused" if fused else "nccl"
+        if args.collectives == "auto":
+            why = shard.fused_self_check(fg, dev)
+            if why is not None:
+                fused, fg = False, None
+                collectives = f"nccl (fused self-check failed: {why})"
+            else:
+                collectives = "fused (self-checked against nccl)"
 
     def run_op(name, op, shp):
         """local compute (our kernels) then the op's one collective (N > 1): NCCL, or
@@ -557,7 +574,7 @@ def run_ours(args) -> None:
             "scaling": "strong", "vs_baseline": None, "dtype": "f32",
             "data": "synthetic: seeded counter-based U[-1,1) fp32 generated in HBM (synth/); paper data sets not shipped",
             "config": {"workload": WORKLOAD_NAME, "parallelism": f"row-sharded x{world}" if world > 1 else "1 GPU",
-                       "collectives": (args.collectives if world > 1 else None),
+                       "collectives": collectives,
                        "l2": "inputs larger than L2: each step streams ~25 GiB; every operand is evicted by the "
                              "following ops before reuse (no flush kernel in the timed region)",
                        "atax_algo": atax_algo, "alpha": ALPHA, "beta": BETA,
@@ -670,9 +687,10 @@ def main():
     ap.add_argument("--test-backend", default="nccl", help=argparse.SUPPRESS)  # tests: gloo with CUDA tensors
     ap.add_argument("--test-one-device", action="store_true", help=argparse.SUPPRESS)  # tests: all ranks on cuda:0
     ap.add_argument("--scale", type=float, default=1.0, help=argparse.SUPPRESS)  # tests: shrink the workload
-    ap.add_argument("--collectives", choices=["nccl", "fused"], default="nccl",
-                    help="N > 1: NCCL collectives (default) or the collective fused into the kernels over "
-                         "NVLink symmetric memory (include/lift_nvlink.h)")
+    ap.add_argument("--collectives", choices=["auto", "nccl", "fused"], default="auto",
+                    help="N > 1: the collective fused into the kernels over NVLink peer memory "
+                         "(include/lift_nvlink.h), or NCCL; auto (default) = fused after a self-check "
+                         "against NCCL on a small problem, else NCCL")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     args = ap.parse_args()
     if args.scale != 1.0:  # test harness only: shrink rows / elements, keep the shapes' columns

@@ -172,6 +172,54 @@ class FusedGroup:
         return self.areas[key]
 
 
+def fused_self_check(fg: FusedGroup, device: torch.device) -> Optional[str]:
+    """Collective: run each fused op once on a small sharded problem with uneven
+    shards and compare it with the same op over torch.distributed collectives
+    (GEMV / GESUMMV bitwise — same rows, same canonical order; dot / ATAX within
+    the north_star tolerance — the two sum the ranks in different orders).
+    Returns None when every rank passed, else a one-line reason (the same
+    verdict on every rank)."""
+    world, rank = _world(fg.group)
+    reason = None
+    try:
+        gen = torch.Generator().manual_seed(20170204)
+        nd, m, n = 10007, 1001, 512
+        xd, yd = torch.rand(nd, generator=gen) - 0.5, torch.rand(nd, generator=gen) - 0.5
+        A, B = torch.rand(m, n, generator=gen) - 0.5, torch.rand(m, n, generator=gen) - 0.5
+        x = (torch.rand(n, generator=gen) - 0.5).to(device)
+        e0, e1 = partition_rows(nd, world, rank)
+        r0, r1 = partition_rows(m, world, rank)
+        xl, yl = xd[e0:e1].to(device), yd[e0:e1].to(device)
+        Al, Bl = A[r0:r1].contiguous().to(device), B[r0:r1].contiguous().to(device)
+
+        def close(a, b, mag):
+            return bool(((a - b).abs() <= 1e-5 * mag + 1e-6).all())
+
+        # every op runs on every rank whatever the earlier verdicts (they are collectives)
+        fails = []
+        got, want = dot_fused(xl, yl, fg), dot(xl, yl, fg.group)
+        if not close(got, want, float((xd * yd).abs().sum())):
+            fails.append(f"dot {float(got)} != {float(want)}")
+        if not torch.equal(gemv_fused(Al, x, m, fg), gemv(Al, x, m, fg.group)):
+            fails.append("gemv all-gather differs")
+        if not torch.equal(gesummv_fused(1.5, Al, 1.2, Bl, x, m, fg), gesummv(1.5, Al, 1.2, Bl, x, m, fg.group)):
+            fails.append("gesummv all-gather differs")
+        got = atax_fused(Al, x, fg, allreduce=True)
+        want = atax(Al, x, fg.group, allreduce=True)
+        if not close(got, want, (A.abs().T @ (A.abs() @ x.abs().cpu())).to(device)):
+            fails.append("atax reduce differs")
+        reason = "; ".join(fails) if fails else None
+        if device.type == "cuda":
+            torch.cuda.synchronize(device)
+    except Exception as e:  # setup or launch failure of the fused path
+        reason = f"{type(e).__name__}: {str(e).splitlines()[0] if str(e) else ''}"
+    flag = torch.tensor([0 if reason is None else 1], device=device, dtype=torch.int32)
+    dist.all_reduce(flag, op=dist.ReduceOp.MAX, group=fg.group)
+    if int(flag.item()) and reason is None:
+        reason = "failed on another rank"
+    return reason
+
+
 def dot_fused(x_loc: torch.Tensor, y_loc: torch.Tensor, fg: FusedGroup, out=None) -> torch.Tensor:
     """dot with the all-reduce inside the kernel: identical bits on every rank."""
     from .nvlink import EXCH_DOT, lift_dot_allreduce

@@ -41,7 +41,7 @@ def test_bench_contract_one_gpu(cuda_device):
     assert d["e2e"]["h2d_bytes_per_step"] > 0 and d["gpu_launches"] == 3 * 5
 
 
-@pytest.mark.parametrize("collectives", ["nccl", "fused"])
+@pytest.mark.parametrize("collectives", ["nccl", "fused", "auto"])
 def test_bench_two_ranks_one_device(cuda_device, collectives):
     cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", "2", "--master-addr",
            "127.0.0.1", "--master-port", str(_port()), "bench.py", "--gpus", "2", "--steps", "2", "--warmup", "3",
@@ -50,4 +50,5 @@ def test_bench_two_ranks_one_device(cuda_device, collectives):
     r = subprocess.run(cmd, cwd=ROOT, capture_output=True, text=True, timeout=900)
     assert r.returncode == 0, (r.stdout[-2000:], r.stderr[-4000:])
     d = _last_json(r.stdout)
-    assert d["n_gpus"] == 2 and d["config"]["collectives"] == collectives and d["value"] > 0
+    want = "fused (self-checked against nccl)" if collectives == "auto" else collectives
+    assert d["n_gpus"] == 2 and d["config"]["collectives"] == want and d["value"] > 0

@@ -132,6 +132,55 @@ def test_sharded_host_logic_gloo(world, m, n):
         assert ok, margin
 
 
+def _selfcheck_worker(rank, world, port, fail_rank, q):
+    sys.path.insert(0, ROOT)
+    try:
+        from paper_conf_cgo_steuwerrd17_b200 import shard
+
+        dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank, world_size=world)
+        ops = _oracle_ops()
+        shard.cuda_ops = lambda: ops  # per-rank compute without a GPU
+        # stand-ins for the fused ops: the collective path itself (so they agree) ...
+        shard.dot_fused = lambda x, y, fg, out=None: shard.dot(x, y, fg.group)
+        shard.gemv_fused = lambda A, x, m, fg, out=None: shard.gemv(A, x, m, fg.group)
+        shard.gesummv_fused = lambda a, A, b, B, x, m, fg, out=None: shard.gesummv(a, A, b, B, x, m, fg.group)
+        shard.atax_fused = lambda A, x, fg, dst=0, allreduce=False, out=None: shard.atax(A, x, fg.group, dst, allreduce)
+        if rank == fail_rank:  # ... except one op on one rank, which returns wrong bits
+            shard.gesummv_fused = lambda a, A, b, B, x, m, fg, out=None: shard.gesummv(a, A, b, B, x, m, fg.group) + 1
+        why = shard.fused_self_check(shard.FusedGroup(), torch.device("cpu"))
+        q.put((rank, why, None))
+        dist.destroy_process_group()
+    except Exception:  # pragma: no cover - reported to the parent
+        import traceback
+
+        q.put((rank, None, traceback.format_exc()))
+
+
+@pytest.mark.parametrize("fail_rank", [-1, 1])
+def test_fused_self_check_verdict_gloo(fail_rank):
+    """bench.py --collectives auto: every rank reaches the same verdict; a
+    mismatch on one rank sends all ranks back to the NCCL path."""
+    world = 2
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_selfcheck_worker, args=(r, world, port, fail_rank, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = {}
+    for _ in range(world):
+        rank, why, err = q.get(timeout=180)
+        assert err is None, err
+        res[rank] = why
+    for p in procs:
+        p.join(timeout=60)
+    if fail_rank < 0:
+        assert res == {0: None, 1: None}
+    else:
+        assert res[fail_rank] == "gesummv all-gather differs"
+        assert res[1 - fail_rank] == "failed on another rank"
+
+
 def test_partition_rows_properties():
     from paper_conf_cgo_steuwerrd17_b200.shard import partition_rows, shard_sizes
 
