@@ -292,9 +292,69 @@ def load_ncu(kernel: str, op_name: str) -> dict:
         return {}
 
 
+def load_table1_ncu(name: str) -> dict:
+    """ncu DRAM % of peak and duration of one Table-1 size (profiles/table1_ncu.json)."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "table1_ncu.json")) as f:
+            return json.load(f).get(name, {})
+    except Exception:
+        return {}
+
+
 def load_traffic(kernel: str, op_name: str):
     """ncu DRAM bytes (read + write) per launch of `kernel` on `op_name`'s shape."""
     return load_ncu(kernel, op_name).get("dram_bytes_per_launch")
+
+
+# The paper's small and large problem sizes (Table 1, L1029-1031: 4K^2 and 8K^2 matrices)
+# plus configs[0]'s dot: measured after the timed region at N = 1 (not part of the step).
+TABLE1 = [
+    ("dot_2^20", "dot", dict(n=1 << 20), "fused"),
+    ("gemv_4096x4096", "gemv", dict(m=4096, n=4096), "fused"),
+    ("gemv_8192x8192", "gemv", dict(m=8192, n=8192), "fused"),
+    ("gesummv_4096x4096", "gesummv", dict(m=4096, n=4096), "fused"),
+    ("gesummv_8192x8192", "gesummv", dict(m=8192, n=8192), "fused"),
+    ("atax_4096x4096", "atax", dict(m=4096, n=4096), "fused"),
+    ("atax_8192x8192", "atax", dict(m=8192, n=8192), "fused"),
+    ("atax_8192x8192_twopass", "atax", dict(m=8192, n=8192), "twopass"),
+]
+
+
+def table1_calls(lift, pool, dot_x, dot_y, dev, l2_bytes):
+    """[(name, op, shape, algo, [call, ...])]: each call reads its own operand slice
+    of the resident buffers (`pool`: flat fp32 >= 2 GiB; dot_x/dot_y: flat fp32), so
+    back-to-back calls stream from HBM (operands rotate over > 2x L2)."""
+    import torch
+
+    out = []
+    for name, op, shp, algo in TABLE1:
+        if op == "dot":
+            n = shp["n"]
+            copies = int(-(-2 * l2_bytes // (8 * n))) + 1
+            res = torch.empty((), device=dev)
+            calls = [(lambda k=k: lift.lift_dot(dot_x[k * n:(k + 1) * n], dot_y[k * n:(k + 1) * n], out=res))
+                     for k in range(copies)]
+        else:
+            m, n = shp["m"], shp["n"]
+            nmat = 2 if op == "gesummv" else 1
+            per = m * n * nmat
+            copies = int(-(-2 * l2_bytes // (4 * per))) + 1
+            if copies * per > pool.numel():
+                raise ValueError("operand pool too small")
+            x = pool[-n:]  # not inside any operand slice read below (copies * per < numel - n)
+            y = torch.empty(n if op == "atax" else m, device=dev)
+
+            def mk(k, op=op, m=m, n=n, per=per, algo=algo, x=x, y=y):
+                A = pool[k * per:k * per + m * n].view(m, n)
+                if op == "gemv":
+                    return lambda: lift.lift_gemv(A, x, out=y)
+                if op == "gesummv":
+                    B = pool[k * per + m * n:(k + 1) * per].view(m, n)
+                    return lambda: lift.lift_gesummv(ALPHA, A, BETA, B, x, out=y)
+                return lambda: lift.lift_atax(A, x, out=y, algo=algo)
+            calls = [mk(k) for k in range(copies)]
+        out.append((name, op, shp, algo, calls))
+    return out
 
 
 def run_ours(args) -> None:
@@ -555,6 +615,39 @@ def run_ours(args) -> None:
                 # against the theoretical DRAM bandwidth the same launch is:
                 "spec_peak": round(spec_peak(), 1), "frac_of_spec_peak": round(achieved / spec_peak(), 4)}
 
+    # the paper's small / large sizes and configs[0]'s dot (N = 1; after the timed region)
+    table1 = None
+    if not distributed and not args.no_table1 and args.scale == 1.0:
+        table1 = {}
+        pool = bufs["gemv_65536x32768"]["A"].view(-1)
+        tcalls = table1_calls(lift, pool, bufs["dot_2^31"]["x"], bufs["dot_2^31"]["y"], dev, l2)
+        for tname, op, shp, algo, calls in tcalls:
+            reps = max(20, len(calls))
+            seq = [calls[j % len(calls)] for j in range(reps)]
+            with torch.cuda.stream(run_stream):
+                g_ = torch.cuda.CUDAGraph()
+                for c in calls:
+                    c()
+                with torch.cuda.graph(g_, stream=run_stream):
+                    for c in seq:
+                        c()
+                g_.replay()
+                torch.cuda.synchronize()
+                s_, e_ = ev(), ev()
+                s_.record()
+                g_.replay()
+                e_.record()
+            torch.cuda.synchronize()
+            ms = s_.elapsed_time(e_) / reps
+            by = alg_bytes(op, shp, algo)
+            gbs = by / (ms * 1e-3) / 1e9
+            nc = load_table1_ncu(tname)
+            table1[tname] = {"us": round(ms * 1e3, 2), "alg_bytes": by, "GB_s": round(gbs, 1),
+                             "frac_of_spec_peak": round(gbs / spec_peak(), 4),
+                             "ncu_dram_pct_of_peak": nc.get("ncu_dram_pct_of_peak"),
+                             "ncu_us": nc.get("us")}
+            del g_
+
     kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 1}[op] for _, op, _, _ in WORKLOAD)
     gpu_launches = kernels_per_step * args.steps
 
@@ -581,7 +674,10 @@ def run_ours(args) -> None:
                        "launch": "cuda-graph of the K timed steps" if use_graph else "eager",
                        "frac_of_peak_per_gpu": round(value / world / peak, 4)},
             "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": gpu_launches,
-            "clocks": sampler.summary(), "ops": ops,
+            "clocks": sampler.summary(), "ops": ops, "table1": table1,
+            "table1_method": "the paper's small/large sizes (Table 1) and configs[0]: >= 20 back-to-back calls "
+                             "in one CUDA graph after the timed region, operands rotated over slices totalling "
+                             "> 2x L2; ncu_* from profiles/table1_ncu.json (tools/table1.py under ncu)",
             "ops_method": "dominant op: events inside the timed steps; others: 10 back-to-back calls after the "
                           "timed region" + (" (one CUDA graph)" if use_graph else "") +
                           ", operands rotated over copies totalling > 2x L2",
@@ -682,6 +778,7 @@ def main():
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--no-e2e", action="store_true", help="skip the end-to-end (host buffers) measurement")
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline oracle timing")
+    ap.add_argument("--no-table1", action="store_true", help="skip the Table-1 sizes block")
     ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--eager", action="store_true", help="launch the timed steps eagerly instead of as a CUDA graph")
     ap.add_argument("--test-backend", default="nccl", help=argparse.SUPPRESS)  # tests: gloo with CUDA tensors

@@ -48,3 +48,15 @@ def test_peaks():
     peak, src = bench.measured_peak()
     assert peak > 1000 and src
     assert abs(bench.spec_peak() - 3996e6 * 2 * 8192 / 8 / 1e9) < 50
+
+
+def test_table1_sizes_cover_paper_and_configs0():
+    """bench.py's table1 block: configs[0]'s dot and the paper's small / large
+    matrix sizes (Table 1: 4K^2 and 8K^2) for every matrix op."""
+    names = {t[0] for t in bench.TABLE1}
+    assert "dot_2^20" in names
+    for op in ("gemv", "gesummv", "atax"):
+        for s in (4096, 8192):
+            assert f"{op}_{s}x{s}" in names
+    cfg0 = json.load(open(os.path.join(ROOT, "BASELINE.json")))["configs"][0]
+    assert "1,048,576" in cfg0 and dict(bench.TABLE1[0][2]) == dict(n=1 << 20)

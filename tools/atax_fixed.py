@@ -1,4 +1,7 @@
-"""Fixed vs per-row cost of the fused ATAX kernel (tuning aid)."""
+"""Fixed vs per-row cost of the fused ATAX kernel (tuning aid).
+
+usage: python tools/atax_fixed.py [n]   (each call reads its own copy of A: HBM, not L2)
+"""
 import os
 import sys
 
@@ -11,18 +14,19 @@ import paper_conf_cgo_steuwerrd17_b200 as lift  # noqa: E402
 from sweep import graph_time  # noqa: E402
 
 dev = torch.device("cuda:0")
-n = 8192
-for m in (148, 296, 592, 1184, 2368, 4736, 8192, 16384):
-    A = synth.torch_matrix_rows(2, n, 0, m, device=dev)
-    x = synth.torch_uniform(0, 0, n, device=dev)
+n = int(sys.argv[1]) if len(sys.argv) > 1 else 8192
+l2 = torch.cuda.get_device_properties(dev).L2_cache_size
+pool = synth.torch_uniform(2, 0, 3 << 28, device=dev)  # 3 GiB
+x = synth.torch_uniform(0, 0, n, device=dev)
+for m in (148, 296, 592, 1184, 2368, 4096, 4736, 8192, 16384):
+    per = m * n
+    copies = min(pool.numel() // per, int(-(-2 * l2 // (4 * per))) + 1)
+    As = [pool[k * per:(k + 1) * per].view(m, n) for k in range(copies)]
+    reps = max(12, copies)
     y = torch.empty(n, device=dev)
     for algo in ("fused", "twopass"):
-        t = graph_time([(lambda: lift.lift_atax(A, x, out=y, algo=algo))] * 10)
-        print(f"{algo:8s} m={m:6d} n={n}: {t:8.2f} us", flush=True)
-    xg = torch.empty(m, device=dev)
-    t = graph_time([(lambda: lift.lift_gemv(A, x, out=xg))] * 10)
-    print(f"gemv     m={m:6d} n={n}: {t:8.2f} us", flush=True)
-    xd = synth.torch_uniform(0, 0, m * n, device=dev)
-    t = graph_time([(lambda: lift.lift_dot(xd, xd))] * 10)
-    print(f"dot      n={m*n:9d}: {t:8.2f} us", flush=True)
-    del A, xd
+        t = graph_time([(lambda A=A: lift.lift_atax(A, x, out=y, algo=algo)) for A in (As * reps)[:reps]])
+        print(f"atax {algo:8s} m={m:6d} n={n}: {t:8.2f} us  {4 * per / t / 1e3:7.1f} GB/s(4mn)", flush=True)
+    yg = torch.empty(m, device=dev)
+    t = graph_time([(lambda A=A: lift.lift_gemv(A, x, out=yg)) for A in (As * reps)[:reps]])
+    print(f"gemv          m={m:6d} n={n}: {t:8.2f} us  {4 * per / t / 1e3:7.1f} GB/s", flush=True)

@@ -18,4 +18,7 @@ for spec in "gemv 4096 4096 auto k_gemv gemv4096" "gesummv 8192 8192 auto k_gemv
   set -- $spec
   timeout 300 ncu --set full --clock-control none --import-source on -k regex:$5 -s 2 -c 1 -o $OUT/full_$6 python tools/one_op.py $1 $2 $3 $4 >> $OUT/ncu_full.log 2>&1
 done
+for name in $(python -c "import bench; print(' '.join(t[0] for t in bench.TABLE1))"); do
+  timeout 300 ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum,gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed --clock-control none -k regex:^k_ --csv --log-file $OUT/table1_$name.csv python tools/table1.py $name >> $OUT/ncu_table1.log 2>&1
+done
 cat $OUT/bench.json

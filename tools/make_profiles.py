@@ -127,6 +127,45 @@ def main(tag, prefix):
                     ent["ncu_duration_us"] = round(float(dur[1].replace(",", "")) * scale, 3)
                 traffic[kern + ":" + label] = ent
     json.dump(traffic, open(tj, "w"), indent=1, sort_keys=True)
+    table1(src, dst, tag, prefix)
+
+
+def table1(src, dst, tag, prefix, calls=4):
+    """ncu launch lists of tools/table1.py NAME (4 calls on distinct operands each)
+    -> profiles/table1_ncu.json (read by bench.py) + profiles/<prefix>_table1_ncu.txt."""
+    files = sorted(f for f in os.listdir(src) if f.startswith("table1_") and f.endswith(".csv"))
+    if not files:
+        return
+    res, lines = {}, [f"# ncu --metrics gpu__time_duration.sum,dram__bytes_*.sum,gpu__dram_throughput.avg."
+                      f"pct_of_peak_sustained_elapsed --clock-control none ({tag}): tools/table1.py NAME,",
+                      "# 4 calls on distinct operands, cold L2 (ncu flushes before every launch); per call: "
+                      "summed kernel time, DRAM bytes, time-weighted DRAM % of peak; median over the calls", ""]
+    for f in files:
+        name = f[len("table1_"):-len(".csv")]
+        try:
+            k = list(load(os.path.join(src, f)).values())
+        except StopIteration:
+            continue
+        if not k or len(k) % calls:
+            continue
+        per = len(k) // calls
+        rows = []
+        for c in range(calls):
+            ks = k[c * per:(c + 1) * per]
+            t = sum(d.get("gpu__time_duration.sum", 0.0) for d in ks)
+            b = sum(d.get("dram__bytes_read.sum", 0.0) + d.get("dram__bytes_write.sum", 0.0) for d in ks)
+            pct = sum(d.get("gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed", 0.0) *
+                      d.get("gpu__time_duration.sum", 0.0) for d in ks) / (t or 1)
+            rows.append((t, b, pct))
+        rows.sort()
+        t, b, pct = rows[len(rows) // 2]
+        res[name] = {"us": round(t / 1e3, 2), "dram_bytes": b, "ncu_dram_pct_of_peak": round(pct, 2),
+                     "kernels_per_call": per}
+        names = ", ".join(sorted({d["name"].split("(")[0].replace("void ", "").split("<")[0] for d in k}))
+        lines.append(f"{name:26s} {t / 1e3:9.2f} us  dram {b / 1e6:9.2f} MB  {b / t if t else 0:8.1f} GB/s  "
+                     f"DRAM {pct:6.2f}% of peak  ({per} kernel(s)/call: {names})")
+    json.dump(res, open(os.path.join(dst, "table1_ncu.json"), "w"), indent=1, sort_keys=True)
+    open(os.path.join(dst, f"{prefix}_table1_ncu.txt"), "w").write("\n".join(lines) + "\n")
 
 
 if __name__ == "__main__":
