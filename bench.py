@@ -332,8 +332,8 @@ def table1_calls(lift, pool, dot_x, dot_y, dev, l2_bytes):
             n = shp["n"]
             copies = int(-(-2 * l2_bytes // (8 * n))) + 1
             res = torch.empty((), device=dev)
-            calls = [(lambda k=k: lift.lift_dot(dot_x[k * n:(k + 1) * n], dot_y[k * n:(k + 1) * n], out=res))
-                     for k in range(copies)]
+            calls = [(lambda xs=dot_x[k * n:(k + 1) * n], ys=dot_y[k * n:(k + 1) * n], res=res:
+                      lift.lift_dot(xs, ys, out=res)) for k in range(copies)]
         else:
             m, n = shp["m"], shp["n"]
             nmat = 2 if op == "gesummv" else 1

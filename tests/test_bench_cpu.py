@@ -60,3 +60,43 @@ def test_table1_sizes_cover_paper_and_configs0():
             assert f"{op}_{s}x{s}" in names
     cfg0 = json.load(open(os.path.join(ROOT, "BASELINE.json")))["configs"][0]
     assert "1,048,576" in cfg0 and dict(bench.TABLE1[0][2]) == dict(n=1 << 20)
+
+
+def test_table1_calls_bind_their_own_operands(monkeypatch):
+    """Every call of every size reads a distinct slice of its own size (no late
+    binding of loop variables), and the slices of one size do not overlap."""
+    import torch
+
+    monkeypatch.setattr(bench, "TABLE1", [("dot_64", "dot", dict(n=64), "fused"),
+                                          ("gemv_8x16", "gemv", dict(m=8, n=16), "fused"),
+                                          ("gesummv_4x8", "gesummv", dict(m=4, n=8), "fused"),
+                                          ("atax_8x4", "atax", dict(m=8, n=4), "twopass")])
+    seen = []
+
+    class Stub:
+        def lift_dot(self, x, y, out):
+            seen.append(("dot", x.numel(), x.data_ptr(), y.numel()))
+
+        def lift_gemv(self, A, x, out):
+            seen.append(("gemv", tuple(A.shape), A.data_ptr(), x.numel()))
+
+        def lift_gesummv(self, a, A, b, B, x, out):
+            assert B.data_ptr() == A.data_ptr() + 4 * A.numel() and a == bench.ALPHA and b == bench.BETA
+            seen.append(("gesummv", tuple(A.shape), A.data_ptr(), x.numel()))
+
+        def lift_atax(self, A, x, out, algo):
+            assert algo == "twopass"
+            seen.append(("atax", tuple(A.shape), A.data_ptr(), x.numel()))
+
+    pool, dx, dy = torch.zeros(1 << 16), torch.zeros(1 << 12), torch.zeros(1 << 12)
+    sets = bench.table1_calls(Stub(), pool, dx, dy, torch.device("cpu"), l2_bytes=1000)
+    for name, op, shp, algo, calls in sets:
+        seen.clear()
+        for c in calls:
+            c()
+        assert len(calls) >= 2 and len({s[2] for s in seen}) == len(calls), name
+        for s in seen:
+            if op == "dot":
+                assert s[1] == s[3] == shp["n"]
+            else:
+                assert s[1] == (shp["m"], shp["n"]) and s[3] == shp["n"]

@@ -27,8 +27,8 @@ for name, op, shp, algo, calls in sets:
     if want is not None:
         if name != want:
             continue
-        for c in calls[:4]:
-            c()
+        for j in range(4):  # (cycles when there are fewer copies; ncu flushes L2 before each launch)
+            calls[j % len(calls)]()
         torch.cuda.synchronize()
         break
     from sweep import graph_time  # noqa: E402
