@@ -108,7 +108,9 @@ def test_dot_full_size_2pow31(cuda_device):
 
 # ===================================================================== GEMV
 GEMV_SHAPES = [(1, 1), (7, 3), (5, 129), (3, 5000), (300, 1000), (1000, 4), (33, 4096), (257, 8192), (4096, 4096),
-               (17, 32768)]
+               (17, 32768),
+               # extremes: x far beyond shared memory (16 MiB rows), ragged wide rows, very tall and skinny
+               (2, 1 << 22), (3, (1 << 20) + 3), (1 << 20, 4), ((1 << 18) + 1, 3)]
 
 
 @pytest.mark.parametrize("m,n", GEMV_SHAPES)
