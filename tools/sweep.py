@@ -71,12 +71,20 @@ def sweep(op, m, n, nsets, ncalls=24):
             continue
         res.append((t, wpr, rg, xs, lb))
         print(f"  wpr={wpr} rg={rg} xs={xs} lb={lb}: {t:8.2f} us  {nbytes / t / 1e3:7.1f} GB/s", flush=True)
-    for blocks in (296, 444, 592, 888, 1184, 1776, 2368):
-        for xs in (0, 1):
-            calls = [mk(A, B, wpr=8, rg=1, xsmem=xs, lb=4, blocks=blocks) for A, B in (sets * ncalls)[:ncalls]]
+    if "--blocks-fine" in sys.argv:  # grid sizes around the row count's divisors x configs
+        grid = [(wpr, rg, blocks) for wpr, rg in ((8, 1), (4, 2), (2, 4), (8, 2), (4, 4))
+                for blocks in (256, 296, 341, 384, 444, 512, 592, 683, 740, 768, 888, 1024, 1184)]
+        xss = (1,)
+    else:
+        grid = [(8, 1, blocks) for blocks in (296, 444, 592, 888, 1184, 1776, 2368)]
+        xss = (0, 1)
+    for wpr, rg, blocks in grid:
+        for xs in xss:
+            calls = [mk(A, B, wpr=wpr, rg=rg, xsmem=xs, lb=4, blocks=blocks) for A, B in (sets * ncalls)[:ncalls]]
             t = graph_time(calls)
-            res.append((t, 8, 1, xs, 4, blocks))
-            print(f"  wpr=8 rg=1 xs={xs} lb=4 blocks={blocks}: {t:8.2f} us  {nbytes / t / 1e3:7.1f} GB/s", flush=True)
+            res.append((t, wpr, rg, xs, 4, blocks))
+            print(f"  wpr={wpr} rg={rg} xs={xs} lb=4 blocks={blocks}: {t:8.2f} us  {nbytes / t / 1e3:7.1f} GB/s",
+                  flush=True)
     res.sort()
     print(f"BEST {op} {m}x{n}: {res[0]}", flush=True)
     del sets
