@@ -580,31 +580,44 @@ def run_ours(args) -> None:
         ops[name] = {"configs_index": cfg, "ms": round(op_ms[i], 4), "alg_bytes": by, "GB_s": round(gbs, 1),
                      "frac_of_peak_per_gpu": round(gbs / world / peak, 4),
                      "ncu_dram_pct_of_peak": load_ncu(kern, name).get("ncu_dram_pct_of_peak")}
-    dom_name, dom_op, dom_shp, _ = WORKLOAD[dom]
-    kernel = {"dot": "k_dot", "gemv": "k_gemv", "gesummv": "k_gemv", "atax": "k_atax_fused"}[dom_op]
-    dom_bytes_rank = alg_bytes(dom_op, dom_shp, atax_algo) / world  # per launch, per rank
-    # at N > 1 the op events include the collective; time the bare kernel once more for the roofline
+    # N > 1: each op's local kernel alone (no collective), so the JSON line separates
+    # compute-only per-rank GB/s from the collective's time (max over ranks, like `ms`)
+    compute_ms = {}
     if distributed:
-        b = bufs[dom_name]
-        kev = [(ev(), ev()) for _ in range(5)]
-        for s, e in kev:
-            s.record()
-            if dom_op == "dot":
+        def local(name, op):
+            b = bufs[name]
+            if op == "dot":
                 lift.lift_dot(b["x"], b["y"], out=b["out"])
-            elif dom_op == "gemv":
+            elif op == "gemv":
                 lift.lift_gemv(b["A"], b["x"], out=b["y_loc"])
-            elif dom_op == "gesummv":
+            elif op == "gesummv":
                 lift.lift_gesummv(ALPHA, b["A"], BETA, b["B"], b["x"], out=b["y_loc"])
             else:
                 lift.lift_atax(b["A"], b["x"], out=b["y"])
-            e.record()
-        torch.cuda.synchronize()
-        kms = max(s.elapsed_time(e) for s, e in kev[2:])
-        t = torch.tensor([kms], device=dev)
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-        kms = float(t[0])
-    else:
-        kms = op_ms[dom]
+
+        for name, op, shp, _ in WORKLOAD:
+            kev = [(ev(), ev()) for _ in range(6)]
+            barrier()
+            for s_, e_ in kev:
+                s_.record()
+                local(name, op)
+                e_.record()
+            torch.cuda.synchronize()
+            kms_ = statistics.median(s_.elapsed_time(e_) for s_, e_ in kev[2:])
+            t = torch.tensor([kms_], device=dev)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+            compute_ms[name] = float(t[0])
+        for i, (name, op, shp, _) in enumerate(WORKLOAD):
+            cm = compute_ms[name]
+            ops[name].update({"compute_ms": round(cm, 4), "collective_ms": round(max(op_ms[i] - cm, 0.0), 4),
+                              "compute_GB_s_per_rank": round(alg_bytes(op, shp, atax_algo) / world / (cm * 1e-3)
+                                                             / 1e9, 1)})
+
+    dom_name, dom_op, dom_shp, _ = WORKLOAD[dom]
+    kernel = {"dot": "k_dot", "gemv": "k_gemv", "gesummv": "k_gemv", "atax": "k_atax_fused"}[dom_op]
+    dom_bytes_rank = alg_bytes(dom_op, dom_shp, atax_algo) / world  # per launch, per rank
+    # at N > 1 the op events include the collective: the roofline takes the bare kernel
+    kms = compute_ms[dom_name] if distributed else op_ms[dom]
     achieved = dom_bytes_rank / (kms * 1e-3) / 1e9
     roofline = {"bound": "hbm", "kernel": kernel, "op": dom_name, "achieved": round(achieved, 1), "peak": peak,
                 "unit": "GB/s", "frac": round(achieved / peak, 4), "traffic": load_traffic(kernel, dom_name),
