@@ -520,6 +520,7 @@ def run_ours(args) -> None:
     # (one CUDA graph at N = 1), so the small ops are not charged for graph event nodes
     # (operands smaller than 2x L2 are rotated over copies so every call streams from HBM)
     op_ms = []
+    op_min_ms = {}
     reps = 10
     l2 = torch.cuda.get_device_properties(dev).L2_cache_size
     for i, (name, op, shp, _) in enumerate(WORKLOAD):
@@ -539,7 +540,9 @@ def run_ours(args) -> None:
             finally:
                 bufs[name] = orig
 
-        s_, e_ = ev(), ev()
+        # `trials` timed repetitions of the `reps` calls: median (reported) and min
+        trials = 5
+        evs = [(ev(), ev()) for _ in range(trials)]
         with torch.cuda.stream(run_stream):
             if use_graph:
                 g_ = torch.cuda.CUDAGraph()
@@ -548,18 +551,21 @@ def run_ours(args) -> None:
                         call(j)
                 g_.replay()
                 barrier()
-                s_.record()
-                g_.replay()
-                e_.record()
+                for s_, e_ in evs:
+                    s_.record()
+                    g_.replay()
+                    e_.record()
             else:
-                barrier()
-                s_.record()
-                for j in range(reps):
-                    call(j)
-                e_.record()
+                for s_, e_ in evs:
+                    barrier()
+                    s_.record()
+                    for j in range(reps):
+                        call(j)
+                    e_.record()
         torch.cuda.synchronize()
         del sets
-        ms = s_.elapsed_time(e_) / reps
+        per = sorted(s_.elapsed_time(e_) / reps for s_, e_ in evs)
+        ms, op_min_ms[name] = statistics.median(per), per[0]
         if distributed:
             t = torch.tensor([ms], device=dev)
             dist.all_reduce(t, op=dist.ReduceOp.MAX)
@@ -577,7 +583,9 @@ def run_ours(args) -> None:
         by = alg_bytes(op, shp, atax_algo)
         gbs = by / (op_ms[i] * 1e-3) / 1e9
         kern = {"dot": "k_dot", "gemv": "k_gemv", "gesummv": "k_gemv", "atax": "k_atax_fused"}[op]
-        ops[name] = {"configs_index": cfg, "ms": round(op_ms[i], 4), "alg_bytes": by, "GB_s": round(gbs, 1),
+        ops[name] = {"configs_index": cfg, "ms": round(op_ms[i], 4),
+                     "ms_min": round(op_min_ms[name], 4) if name in op_min_ms else None,
+                     "alg_bytes": by, "GB_s": round(gbs, 1),
                      "frac_of_peak_per_gpu": round(gbs / world / peak, 4),
                      "ncu_dram_pct_of_peak": load_ncu(kern, name).get("ncu_dram_pct_of_peak")}
     # N > 1: each op's local kernel alone (no collective), so the JSON line separates
@@ -646,16 +654,19 @@ def run_ours(args) -> None:
                         c()
                 g_.replay()
                 torch.cuda.synchronize()
-                s_, e_ = ev(), ev()
-                s_.record()
-                g_.replay()
-                e_.record()
+                evs = [(ev(), ev()) for _ in range(5)]
+                for s_, e_ in evs:
+                    s_.record()
+                    g_.replay()
+                    e_.record()
             torch.cuda.synchronize()
-            ms = s_.elapsed_time(e_) / reps
+            per = sorted(s_.elapsed_time(e_) / reps for s_, e_ in evs)
+            ms = statistics.median(per)
             by = alg_bytes(op, shp, algo)
             gbs = by / (ms * 1e-3) / 1e9
             nc = load_table1_ncu(tname)
-            table1[tname] = {"us": round(ms * 1e3, 2), "alg_bytes": by, "GB_s": round(gbs, 1),
+            table1[tname] = {"us": round(ms * 1e3, 2), "us_min": round(per[0] * 1e3, 2), "alg_bytes": by,
+                             "GB_s": round(gbs, 1),
                              "frac_of_spec_peak": round(gbs / spec_peak(), 4),
                              "ncu_dram_pct_of_peak": nc.get("ncu_dram_pct_of_peak"),
                              "ncu_us": nc.get("us")}
@@ -690,10 +701,12 @@ def run_ours(args) -> None:
             "clocks": sampler.summary(), "ops": ops, "table1": table1,
             "table1_method": "the paper's small/large sizes (Table 1) and configs[0]: >= 20 back-to-back calls "
                              "in one CUDA graph after the timed region, operands rotated over slices totalling "
-                             "> 2x L2; ncu_* from profiles/table1_ncu.json (tools/table1.py under ncu)",
+                             "> 2x L2; us = median of 5 replays, us_min their minimum; ncu_* from "
+                             "profiles/table1_ncu.json (tools/table1.py under ncu)",
             "ops_method": "dominant op: events inside the timed steps; others: 10 back-to-back calls after the "
                           "timed region" + (" (one CUDA graph)" if use_graph else "") +
-                          ", operands rotated over copies totalling > 2x L2",
+                          ", operands rotated over copies totalling > 2x L2; ms = median of 5 such runs, "
+                          "ms_min their minimum",
         }
         print(json.dumps(line), flush=True)
     if distributed:
