@@ -285,6 +285,7 @@ constexpr size_t kFusedStageTarget = 32 * 1024;
 constexpr size_t kFusedRingTarget = 112 * 1024;
 constexpr int kFusedL2Ahead = 0;
 constexpr int kFusedCyclic = 1;
+constexpr int kFusedXsmemQc = 8;  // qc at which x moves from registers to shared memory
 
 static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}) {
     if (n <= 0 || n % 4 != 0) return false;
@@ -301,12 +302,15 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
     int64_t nst = (int64_t)((kFusedRingTarget + stage / 2) / stage);
     if (nst < 2) nst = 2;
     if (nst > kFusedMaxStages) nst = kFusedMaxStages;
-    while (nst > 2 && hdr + (size_t)nst * stage > (size_t)kFusedSmemBudget) --nst;
+    // 8 float4 columns per thread: x lives in shared memory after the ring instead of
+    // registers (x, y, and two steps of a row would need all 128 registers)
+    const size_t xs_bytes = qc >= kFusedXsmemQc ? (size_t)n * 4 : 0;
+    while (nst > 2 && hdr + (size_t)nst * stage + xs_bytes > (size_t)kFusedSmemBudget) --nst;
     if (tune.nst != 0) {  // explicit ring depth (lift_tuning.h): must fit as given
         if (tune.nst < 2 || tune.nst > kFusedMaxStages) return false;
         nst = tune.nst;
     }
-    if (hdr + (size_t)nst * stage > (size_t)kFusedSmemBudget) return false;
+    if (hdr + (size_t)nst * stage + xs_bytes > (size_t)kFusedSmemBudget) return false;
     if (tune.l2a < -1 || tune.l2a > 64 || tune.cyc < -1 || tune.cyc > 1) return false;
     p->qc = qc;
     p->cr = cr;
@@ -316,7 +320,7 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
     p->hdr = hdr;
     // the drained ring is reused for the final column-sum tile partials
     const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
-    p->smem = hdr + (ring > tile ? ring : tile);
+    p->smem = hdr + (ring > tile ? ring : tile) + xs_bytes;
     return true;
 }
 
@@ -460,12 +464,17 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         for (int i = 0; i < l2a; ++i) prefetch_stage(nst + i);
     }
 
-    float4 xr[QC], yr[QC];
+    constexpr bool XS = QC >= kFusedXsmemQc;  // x in shared memory (after the ring) instead of registers
+    float4 xr[XS ? 1 : QC], yr[QC];
     const float4 *x4 = reinterpret_cast<const float4 *>(x);
+    float4 *xs4 = reinterpret_cast<float4 *>(stage0 + (size_t)nst * stage_floats);
+    if constexpr (XS) {
+        for (int64_t c = tid; c < nv; c += kFusedThreads) xs4[c] = ld_ro4(x4 + c);  // visible after the loop's barrier
+    }
 #pragma unroll
     for (int q = 0; q < QC; ++q) {
         const int64_t c = tid + (int64_t)kFusedThreads * q;
-        xr[q] = c < nv ? ld_ro4(x4 + c) : zero4();
+        if constexpr (!XS) xr[q] = c < nv ? ld_ro4(x4 + c) : zero4();
         yr[q] = zero4();
     }
     // Software-pipelined over steps (one step = one stage of CR rows): iteration
@@ -510,7 +519,14 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
             for (int i = 0; i < CR; ++i) {
                 float4 acc = zero4();
 #pragma unroll
-                for (int q = 0; q < QC; ++q) fma4(acc, a[i][q], xr[q]);
+                for (int q = 0; q < QC; ++q) {
+                    if constexpr (XS) {
+                        const int64_t c = tid + (int64_t)kFusedThreads * q;
+                        fma4(acc, a[i][q], c < nv ? xs4[c] : zero4());
+                    } else {
+                        fma4(acc, a[i][q], xr[q]);
+                    }
+                }
                 d[i] = hsum4(acc);
             }
 #pragma unroll

@@ -343,7 +343,7 @@ def test_atax_fused_tuning(cuda_device):
                     try:
                         got = lift.lift_atax_fused_tuned(A, x, nst=nst, l2_ahead=l2a, cyclic=cyc)
                     except lift.LiftError:  # ring does not fit the shared-memory budget
-                        assert n >= 8192 and nst >= 5, (m, n, nst)
+                        assert n > 8192 and nst >= 3, (m, n, nst)  # 64 KiB rows + x in smem: 2 stages max
                         continue
                     assert torch.equal(got, base), (m, n, cyc, nst, l2a)
         assert hits >= 1
