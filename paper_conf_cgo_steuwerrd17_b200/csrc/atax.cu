@@ -132,42 +132,49 @@ template <int VEC, int TPB, int UR>
 __global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int64_t lda, int S,
                                                    const float *__restrict__ A, const float *__restrict__ t,
                                                    float *__restrict__ P) {
-    extern __shared__ float ts[];  // t for this row split (toLocal)
     using V = typename std::conditional<VEC == 4, float4, float>::type;
     const int s = blockIdx.y;
     const int64_t r0 = m * s / S, r1 = m * (s + 1) / S;
-    for (int64_t r = r0 + threadIdx.x; r < r1; r += TPB) ts[r - r0] = __ldg(t + r);
-    __syncthreads();
     const int64_t nv = n / VEC;
     const int64_t c = (int64_t)blockIdx.x * TPB + threadIdx.x;
     if (c >= nv) return;
     const int64_t ldv = lda / VEC;  // row stride in vectors
-    const V *A4 = reinterpret_cast<const V *>(A);
+    const V *AV = reinterpret_cast<const V *>(A);
     V acc;
     if constexpr (VEC == 4) acc = zero4(); else acc = 0.f;
-    int64_t r = r0;
-    for (; r + UR <= r1; r += UR) {
-        V a[UR];
+    // rows r0, r0+1, ... in order (reduceSeq), UR rows per batch, the next batch's
+    // loads issued before this one is consumed; a ragged last batch is predicated
+    V cur[UR], nxt[UR];
+    float tc[UR], tn[UR];  // t_i for the batch (same address across the block: broadcast)
+    auto load = [&](int64_t rb, V(&a)[UR], float(&tt)[UR]) {
 #pragma unroll
         for (int u = 0; u < UR; ++u) {
-            if constexpr (VEC == 4)
-                a[u] = ld_stream4(A4 + (r + u) * ldv + c);
-            else
-                a[u] = ld_stream1(A + (r + u) * lda + c);
+            if (rb + u < r1) {
+                if constexpr (VEC == 4)
+                    a[u] = ld_stream4(AV + (rb + u) * ldv + c);
+                else
+                    a[u] = ld_stream1(A + (rb + u) * lda + c);
+                tt[u] = __ldg(t + rb + u);
+            }
+        }
+    };
+    if (r0 < r1) load(r0, cur, tc);
+    for (int64_t r = r0; r < r1; r += UR) {
+        if (r + UR < r1) load(r + UR, nxt, tn);
+#pragma unroll
+        for (int u = 0; u < UR; ++u) {
+            if (r + u < r1) {
+                if constexpr (VEC == 4)
+                    fma4s(acc, cur[u], tc[u]);
+                else
+                    acc = __fmaf_rn(cur[u], tc[u], acc);
+            }
         }
 #pragma unroll
         for (int u = 0; u < UR; ++u) {
-            if constexpr (VEC == 4)
-                fma4s(acc, a[u], ts[r + u - r0]);
-            else
-                acc = __fmaf_rn(a[u], ts[r + u - r0], acc);
+            cur[u] = nxt[u];
+            tc[u] = tn[u];
         }
-    }
-    for (; r < r1; ++r) {
-        if constexpr (VEC == 4)
-            fma4s(acc, ld_stream4(A4 + r * ldv + c), ts[r - r0]);
-        else
-            acc = __fmaf_rn(ld_stream1(A + r * lda + c), ts[r - r0], acc);
     }
     reinterpret_cast<V *>(P)[(int64_t)s * nv + c] = acc;
 }
@@ -180,29 +187,21 @@ static cudaError_t column_pass(const DeviceInfo &d, int64_t m, int64_t n, int64_
     constexpr int TPB = 256;
     const int64_t nv = vec ? n / 4 : n;
     const int64_t cblocks = (nv + TPB - 1) / TPB;
-    // about 8 resident 256-thread blocks per SM
-    int64_t S = ((int64_t)d.sms * 8 + cblocks - 1) / cblocks;
+    // one resident wave: column blocks x row splits = SMs x blocks per SM
+    int per_sm = 0;
+    cudaError_t e = vec ? cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_atax_cols<4, TPB, 8>, TPB, 0)
+                        : cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_atax_cols<1, TPB, 8>, TPB, 0);
+    if (e != cudaSuccess) return e;
+    if (per_sm < 1) per_sm = 1;
+    int64_t S = (int64_t)d.sms * per_sm / cblocks;
     if (S > kMaxSplits) S = kMaxSplits;
     if (S > m) S = m;
     if (S < 1) S = 1;
-    const size_t smem = (size_t)((m + S - 1) / S + 1) * 4;
     dim3 grid((unsigned)cblocks, (unsigned)S);
-    cudaError_t e;
-    if (vec) {
-        auto k = k_atax_cols<4, TPB, 8>;
-        if (smem > 48 * 1024) {
-            e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-            if (e != cudaSuccess) return e;
-        }
-        k<<<grid, TPB, smem, s>>>(m, n, lda, (int)S, A, t, P);
-    } else {
-        auto k = k_atax_cols<1, TPB, 8>;
-        if (smem > 48 * 1024) {
-            e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-            if (e != cudaSuccess) return e;
-        }
-        k<<<grid, TPB, smem, s>>>(m, n, lda, (int)S, A, t, P);
-    }
+    if (vec)
+        k_atax_cols<4, TPB, 8><<<grid, TPB, 0, s>>>(m, n, lda, (int)S, A, t, P);
+    else
+        k_atax_cols<1, TPB, 8><<<grid, TPB, 0, s>>>(m, n, lda, (int)S, A, t, P);
     e = cudaGetLastError();
     if (e != cudaSuccess) return e;
     return vec ? run_colsum<4>((int)S, n, P, y, s, alpha, beta, axpby)
