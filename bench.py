@@ -244,7 +244,22 @@ def cpu_baseline(min_seconds: float = 10.0) -> dict:
         ts.append(time.perf_counter() - t1)
     return {"value": round(gbs, 3), "unit": "GB/s", "cores": th, "kind": "oracle",
             "sample": desc + f"; {passes} passes in {el:.1f} s",
-            "configs0_dot_2^20_ms": round(1e3 * sorted(ts)[2], 3)}
+            "configs0_dot_2^20_ms": round(1e3 * sorted(ts)[2], 3), "host": host_info()}
+
+
+def host_info() -> dict:
+    """The host the CPU legs ran on (count, affinity, model name)."""
+    model = None
+    try:
+        with open("/proc/cpuinfo") as f:
+            model = next((l.split(":", 1)[1].strip() for l in f if l.startswith("model name")), None)
+    except OSError:
+        pass
+    try:
+        aff = len(os.sched_getaffinity(0))
+    except AttributeError:  # pragma: no cover
+        aff = None
+    return {"cpu_count": os.cpu_count(), "affinity": aff, "model": model}
 
 
 def run_reference(args) -> None:
@@ -267,7 +282,8 @@ def run_reference(args) -> None:
         "ms_per_step": round(1e3 * el / args.steps, 3), "higher_is_better": True, "scaling": "strong",
         "vs_baseline": None, "dtype": "f64", "data": "synthetic (seeded counter-based U[-1,1) fp32 inputs)",
         "config": {"workload": WORKLOAD_NAME, "sample": "bounded (see cpu_baseline.sample)"},
-        "cpu_baseline": {"value": round(gbs, 3), "unit": "GB/s", "cores": th, "kind": "oracle", "sample": desc},
+        "cpu_baseline": {"value": round(gbs, 3), "unit": "GB/s", "cores": th, "kind": "oracle", "sample": desc,
+                         "host": host_info()},
         "e2e": {"value": round(gbs, 3), "unit": "GB/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -691,6 +707,7 @@ def run_ours(args) -> None:
             "scaling": "strong", "vs_baseline": None, "dtype": "f32",
             "data": "synthetic: seeded counter-based U[-1,1) fp32 generated in HBM (synth/); paper data sets not shipped",
             "config": {"workload": WORKLOAD_NAME, "parallelism": f"row-sharded x{world}" if world > 1 else "1 GPU",
+                       "gpu": torch.cuda.get_device_name(dev),
                        "collectives": collectives,
                        "l2": "inputs larger than L2: each step streams ~25 GiB; every operand is evicted by the "
                              "following ops before reuse (no flush kernel in the timed region)",
