@@ -102,7 +102,19 @@ def alg_bytes(op: str, shp: dict, atax_algo: str = "fused") -> int:
     """Algorithmic HBM bytes of one op on the GLOBAL problem."""
     if op == "dot":
         return 8 * shp["n"] + 4
+    if op == "partial_dot":  # NEXT-3: z[n/128] written (Listing 1)
+        return 8 * shp["n"] + 4 * (shp["n"] // 128)
+    if op == "dot_listing1":  # NEXT-3 iterated to one value: the later stages re-read the partials
+        n, by, ln = shp["n"], 8 * shp["n"], -(-shp["n"] // 128)
+        by += 4 * ln
+        while ln > 1:
+            ln2 = -(-ln // 128)
+            by += 4 * ln + 4 * ln2
+            ln = ln2
+        return by
     m, n = shp["m"], shp["n"]
+    if op == "sgemv_t":  # NEXT-4: y[n] = alpha A^T x[m] + beta y (y read when beta != 0)
+        return 4 * m * n + 4 * m + 4 * n * (2 if shp.get("beta", 0.0) != 0.0 else 1)
     if op == "gemv":
         return 4 * m * n + 4 * (m + n)
     if op == "gesummv":
@@ -333,6 +345,12 @@ TABLE1 = [
     ("atax_4096x4096", "atax", dict(m=4096, n=4096), "fused"),
     ("atax_8192x8192", "atax", dict(m=8192, n=8192), "fused"),
     ("atax_8192x8192_twopass", "atax", dict(m=8192, n=8192), "twopass"),
+    # SURVEY.md §8f NEXT-3 (Listing 1 literally) and NEXT-4 (BLAS SGEMV, transposed)
+    ("partial_dot_2^20", "partial_dot", dict(n=1 << 20), None),
+    ("partial_dot_2^28", "partial_dot", dict(n=1 << 28), None),
+    ("dot_listing1_2^28", "dot_listing1", dict(n=1 << 28), None),
+    ("sgemv_t_8192x8192", "sgemv_t", dict(m=8192, n=8192, beta=0.0), None),
+    ("sgemv_t_8192x8192_beta", "sgemv_t", dict(m=8192, n=8192, beta=0.5), None),
 ]
 
 
@@ -344,12 +362,19 @@ def table1_calls(lift, pool, dot_x, dot_y, dev, l2_bytes):
 
     out = []
     for name, op, shp, algo in TABLE1:
-        if op == "dot":
+        if op in ("dot", "partial_dot", "dot_listing1"):
             n = shp["n"]
             copies = int(-(-2 * l2_bytes // (8 * n))) + 1
-            res = torch.empty((), device=dev)
-            calls = [(lambda xs=dot_x[k * n:(k + 1) * n], ys=dot_y[k * n:(k + 1) * n], res=res:
-                      lift.lift_dot(xs, ys, out=res)) for k in range(copies)]
+            if copies * n > dot_x.numel():
+                raise ValueError("dot operands too small")
+            if op == "partial_dot":
+                res = torch.empty(n // 128, device=dev)
+                fn = lift.lift_partial_dot
+            else:
+                res = torch.empty((), device=dev)
+                fn = lift.lift_dot if op == "dot" else lift.lift_dot_listing1
+            calls = [(lambda xs=dot_x[k * n:(k + 1) * n], ys=dot_y[k * n:(k + 1) * n], res=res, fn=fn:
+                      fn(xs, ys, out=res)) for k in range(copies)]
         else:
             m, n = shp["m"], shp["n"]
             nmat = 2 if op == "gesummv" else 1
@@ -357,8 +382,10 @@ def table1_calls(lift, pool, dot_x, dot_y, dev, l2_bytes):
             copies = int(-(-2 * l2_bytes // (4 * per))) + 1
             if copies * per > pool.numel():
                 raise ValueError("operand pool too small")
-            x = pool[-n:]  # not inside any operand slice read below (copies * per < numel - n)
-            y = torch.empty(n if op == "atax" else m, device=dev)
+            x = pool[-(m if op == "sgemv_t" else n):]  # not inside any operand slice read below (copies * per < numel - n)
+            y = torch.empty(n if op in ("atax", "sgemv_t") else m, device=dev)
+            if op == "sgemv_t":
+                y.fill_(0.5)
 
             def mk(k, op=op, m=m, n=n, per=per, algo=algo, x=x, y=y):
                 A = pool[k * per:k * per + m * n].view(m, n)
@@ -367,6 +394,10 @@ def table1_calls(lift, pool, dot_x, dot_y, dev, l2_bytes):
                 if op == "gesummv":
                     B = pool[k * per + m * n:(k + 1) * per].view(m, n)
                     return lambda: lift.lift_gesummv(ALPHA, A, BETA, B, x, out=y)
+                if op == "sgemv_t":
+                    # beta != 0 reads and rewrites y (|beta| < 1 keeps repeated calls bounded)
+                    bt = shp["beta"]
+                    return lambda: lift.lift_sgemv(1.0 if bt == 0.0 else ALPHA, A, x, bt, y=y, trans=True)
                 return lambda: lift.lift_atax(A, x, out=y, algo=algo)
             calls = [mk(k) for k in range(copies)]
         out.append((name, op, shp, algo, calls))

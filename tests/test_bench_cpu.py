@@ -30,6 +30,14 @@ def test_algorithmic_bytes():
     assert bench.alg_bytes("gesummv", dict(m=8192, n=8192)) == 536936448
     assert bench.alg_bytes("atax", dict(m=8192, n=8192)) == 268500992
     assert bench.alg_bytes("atax", dict(m=8192, n=8192), "twopass") == 537001984
+    # NEXT-3: x, y read, z[n/128] written; iterated: 2^28 -> 2^21 -> 16384 -> 128 -> 1 partials
+    assert bench.alg_bytes("partial_dot", dict(n=1 << 20)) == 8 * (1 << 20) + 4 * 8192
+    stages = [1 << 21, 1 << 14, 1 << 7, 1]
+    assert bench.alg_bytes("dot_listing1", dict(n=1 << 28)) == (
+        8 * (1 << 28) + 4 * stages[0] + sum(4 * a + 4 * b for a, b in zip(stages, stages[1:])))
+    # NEXT-4 transposed SGEMV: A, x[m] read, y[n] written (and read when beta != 0)
+    assert bench.alg_bytes("sgemv_t", dict(m=8192, n=4096, beta=0.0)) == 4 * 8192 * 4096 + 4 * 8192 + 4 * 4096
+    assert bench.alg_bytes("sgemv_t", dict(m=8192, n=4096, beta=0.5)) == 4 * 8192 * 4096 + 4 * 8192 + 8 * 4096
 
 
 def test_reference_arm_contract_line():
@@ -70,7 +78,10 @@ def test_table1_calls_bind_their_own_operands(monkeypatch):
     monkeypatch.setattr(bench, "TABLE1", [("dot_64", "dot", dict(n=64), "fused"),
                                           ("gemv_8x16", "gemv", dict(m=8, n=16), "fused"),
                                           ("gesummv_4x8", "gesummv", dict(m=4, n=8), "fused"),
-                                          ("atax_8x4", "atax", dict(m=8, n=4), "twopass")])
+                                          ("atax_8x4", "atax", dict(m=8, n=4), "twopass"),
+                                          ("partial_dot_256", "partial_dot", dict(n=256), None),
+                                          ("dot_listing1_128", "dot_listing1", dict(n=128), None),
+                                          ("sgemv_t_8x4", "sgemv_t", dict(m=8, n=4, beta=0.5), None)])
     seen = []
 
     class Stub:
@@ -88,6 +99,17 @@ def test_table1_calls_bind_their_own_operands(monkeypatch):
             assert algo == "twopass"
             seen.append(("atax", tuple(A.shape), A.data_ptr(), x.numel()))
 
+        def lift_partial_dot(self, x, y, out):
+            assert out.numel() == x.numel() // 128
+            seen.append(("partial_dot", x.numel(), x.data_ptr(), y.numel()))
+
+        def lift_dot_listing1(self, x, y, out):
+            seen.append(("dot_listing1", x.numel(), x.data_ptr(), y.numel()))
+
+        def lift_sgemv(self, alpha, A, x, beta, y, trans):
+            assert trans and beta == 0.5 and y.numel() == A.shape[1]
+            seen.append(("sgemv_t", tuple(A.shape), A.data_ptr(), x.numel()))
+
     pool, dx, dy = torch.zeros(1 << 16), torch.zeros(1 << 12), torch.zeros(1 << 12)
     sets = bench.table1_calls(Stub(), pool, dx, dy, torch.device("cpu"), l2_bytes=1000)
     for name, op, shp, algo, calls in sets:
@@ -96,7 +118,9 @@ def test_table1_calls_bind_their_own_operands(monkeypatch):
             c()
         assert len(calls) >= 2 and len({s[2] for s in seen}) == len(calls), name
         for s in seen:
-            if op == "dot":
+            if op in ("dot", "partial_dot", "dot_listing1"):
                 assert s[1] == s[3] == shp["n"]
+            elif op == "sgemv_t":
+                assert s[1] == (shp["m"], shp["n"]) and s[3] == shp["m"]
             else:
                 assert s[1] == (shp["m"], shp["n"]) and s[3] == shp["n"]

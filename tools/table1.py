@@ -19,8 +19,8 @@ import paper_conf_cgo_steuwerrd17_b200 as lift  # noqa: E402
 dev = torch.device("cuda:0")
 l2 = torch.cuda.get_device_properties(dev).L2_cache_size
 pool = synth.torch_uniform(synth.SEED_A, 0, (3 << 30) // 4 * 1, device=dev)  # 3 GiB of operands
-dx = synth.torch_uniform(synth.SEED_X, 0, 40 << 20, device=dev)
-dy = synth.torch_uniform(synth.SEED_Y, 0, 40 << 20, device=dev)
+dx = synth.torch_uniform(synth.SEED_X, 0, 1 << 29, device=dev)  # 2 GiB: two copies of the 2^28 dots
+dy = synth.torch_uniform(synth.SEED_Y, 0, 1 << 29, device=dev)
 sets = bench.table1_calls(lift, pool, dx, dy, dev, l2)
 want = sys.argv[1] if len(sys.argv) > 1 else None
 for name, op, shp, algo, calls in sets:
