@@ -339,7 +339,8 @@ bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
 // the order depends only on S.
 template <int IF /* loads in flight per thread */>
 __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__restrict__ P, float *__restrict__ y,
-                                             int64_t c0, int64_t c1, float4 *part /* smem [32][16] */) {
+                                             int64_t c0, int64_t c1, float4 *part /* smem [32][16] */,
+                                             bool discard /* c0, c1 on 128-byte lines: drop them after use */) {
     constexpr int CW = 16, SPL = 32;
     const int tid = threadIdx.x;
     const int col = tid % CW, sp = tid / CW;
@@ -368,7 +369,13 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
             }
         }
         part[sp * CW + col] = acc;
-        __syncthreads();
+        __syncthreads();  // every load of this pass has been consumed
+        if (discard) {    // its lines (2 per row) of every partial row are dead now
+            const int64_t e = cb + CW < c1 ? cb + CW : c1;
+            const int nl = (int)((e - cb + 7) / 8);
+            for (int k = tid; k < S * nl; k += kFusedThreads)
+                discard_l2_line(P4 + (int64_t)(k / nl) * nv + cb + 8 * (k % nl));
+        }
         if (tid < CW && c < c1) {
             float comp[4][SPL];
 #pragma unroll
@@ -384,6 +391,15 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
         }
         __syncthreads();
     }
+}
+
+// The fused kernel's partial rows may be discarded from L2 after their last
+// read only when every row is a whole number of 128-byte lines (no line shared
+// by two rows).  Measured (profiles/r01u_atax_discard.txt): fused ATAX 8192^2
+// 45.4 -> 44.3 us, 16384x8192 82.4 -> 81.4 us; the two-pass column sum and
+// the transposed SGEMV gained nothing from it and do not discard.
+static bool rows_are_lines(const float *P, int64_t n) {
+    return n % 32 == 0 && (reinterpret_cast<uintptr_t>(P) & 127) == 0;
 }
 
 // One-shot grid barrier for a cooperative launch (all blocks co-resident).
@@ -417,7 +433,7 @@ template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
     k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
                  float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar, Exch ex,
-                 int dst, int l2a, int cyc) {
+                 int dst, int l2a, int cyc, bool discard_partials) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
@@ -581,9 +597,14 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     // ---- second stage in the same launch: grid barrier, then every block sums
     // a slice of the columns over all G partial rows in a fixed order ----
     grid_barrier(gbar);
-    // every block sums its own slice of columns (the drained ring holds the split sums)
-    const int64_t c0 = nv * blockIdx.x / gridDim.x, c1 = nv * (blockIdx.x + 1) / gridDim.x;
-    colsum_slice<8>((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0));
+    // every block sums its own slice of columns (the drained ring holds the split sums);
+    // when the partial rows are whole 128-byte lines the slices are too, and each block
+    // discards the lines it has read (no DRAM write-back of dead partials)
+    const bool lines = discard_partials;
+    const int64_t unit = lines ? 8 : 1, nu = (nv + unit - 1) / unit;
+    int64_t c0 = unit * (nu * blockIdx.x / gridDim.x), c1 = unit * (nu * (blockIdx.x + 1) / gridDim.x);
+    if (c1 > nv) c1 = nv;
+    colsum_slice<8>((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0), lines);
     if (ex.world == 0) {
         grid_depart(gbar);
         return;
@@ -645,7 +666,8 @@ static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const flo
     attr[0].val.cooperative = 1;
     cfg.attrs = attr;
     cfg.numAttrs = cooperative ? 1 : 0;
-    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.l2a, p.cyc);
+    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.l2a, p.cyc,
+                              rows_are_lines(P, n));
 }
 
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)

@@ -396,6 +396,49 @@ def test_atax_deterministic(cuda_device):
             assert torch.equal(lift.lift_atax(A, x, algo=algo), a)
 
 
+@pytest.mark.parametrize("m,n", [(3000, 4096), (8192, 8192), (700, 16384), (513, 96)])
+def test_partial_rows_discard_is_invisible(cuda_device, m, n):
+    """The partial-sum rows are dropped from L2 after their last read
+    (discard.global.L2) only when each row is whole 128-byte lines; a
+    workspace offset by 16 bytes turns that off.  Results must be bitwise the
+    same either way, and across repeated calls that rewrite discarded lines
+    (fused ATAX; the two-pass ATAX and the transposed SGEMV, whose column sums
+    do not discard, are checked the same way)."""
+    L = lift.lib()
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    xt = synth.torch_uniform(synth.SEED_Y, 0, m, device=cuda_device)
+    stream = torch.cuda.current_stream(cuda_device).cuda_stream
+
+    def ws_pair(nbytes):
+        a = torch.zeros(nbytes + 512, dtype=torch.uint8, device=cuda_device)
+        b = torch.zeros(nbytes + 512, dtype=torch.uint8, device=cuda_device)
+        return a, b[16:]  # 256-byte aligned base (discard on) / 16-byte offset (off)
+
+    for algo in (lift.LIFT_ATAX_FUSED, lift.LIFT_ATAX_TWOPASS):
+        nb = L.lift_atax_workspace_bytes(m, n)
+        outs = []
+        for ws in ws_pair(nb):
+            for _ in range(3):
+                y = torch.empty(n, device=cuda_device)
+                lift.check(L.lift_atax_algo_run(algo, m, n, A.data_ptr(), x.data_ptr(), y.data_ptr(),
+                                                ws.data_ptr(), nb, stream))
+                outs.append(y)
+        assert all(torch.equal(o, outs[0]) for o in outs), algo
+    nb = L.lift_sgemv_workspace_bytes(0, 1, m, n)
+    outs = []
+    for ws in ws_pair(nb):
+        for _ in range(3):
+            y = torch.full((n,), 0.25, device=cuda_device)
+            lift.check(L.lift_sgemv(0, 1, m, n, 1.5, A.data_ptr(), n, xt.data_ptr(), 0.5, y.data_ptr(),
+                                    ws.data_ptr(), nb, stream))
+            outs.append(y)
+    assert all(torch.equal(o, outs[0]) for o in outs)
+    if m * n <= 1 << 24:
+        ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+        assert_tol(lift.lift_atax(A, x, algo="fused").cpu().numpy(), ref, mag, "atax after discards")
+
+
 def test_atax_unaligned(cuda_device):
     m, n = 50, 301
     buf = dev_np(rand(2, (m * n + 1,)), cuda_device)

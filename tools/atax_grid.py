@@ -51,7 +51,9 @@ for m, n, sets in ((8192, 8192, 3), (4096, 4096, 8), (16384, 8192, 2)):
     print(f"atax {m}x{n} library (cooperative, {sms} blocks): {t:8.2f} us  {by / t / 1e3:8.1f} GB/s", flush=True)
     for blocks in (sms, 144, 136, 128, 120, 112, 96, 74):
         got = nvlink.lift_atax_reduce(As[0], x, ex, dst=0, blocks=blocks, workspace=ws)
-        assert torch.allclose(got, ref, rtol=1e-4, atol=1e-3), blocks
+        # a different block count sums in a different order: compare at the scale of y
+        # (tools/atax_blocks_check.py checks each against fp64 with the north_star tolerance)
+        assert (got - ref).abs().max() <= 1e-5 * ref.abs().max(), blocks
         calls = [(lambda A=A, b=blocks: nvlink.lift_atax_reduce(A, x, ex, dst=0, out=y, blocks=b, workspace=ws))
                  for A in (As * 30)[:30]]
         t = time_calls(calls)
