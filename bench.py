@@ -346,6 +346,7 @@ TABLE1 = [
     ("atax_8192x8192", "atax", dict(m=8192, n=8192), "fused"),
     ("atax_8192x8192_twopass", "atax", dict(m=8192, n=8192), "twopass"),
     # SURVEY.md §8f NEXT-3 (Listing 1 literally) and NEXT-4 (BLAS SGEMV, transposed)
+    ("dot_2^28", "dot", dict(n=1 << 28), "fused"),  # k_dot at the size of the NEXT-3 rows below
     ("partial_dot_2^20", "partial_dot", dict(n=1 << 20), None),
     ("partial_dot_2^28", "partial_dot", dict(n=1 << 28), None),
     ("dot_listing1_2^28", "dot_listing1", dict(n=1 << 28), None),
