@@ -405,14 +405,22 @@ static bool rows_are_lines(const float *P, int64_t n) {
 // One-shot grid barrier for a cooperative launch (all blocks co-resident).
 // gbar[0] counts arrivals, gbar[1] departures; the last block to depart
 // re-arms both to zero for the next launch on this workspace.
+// Arrival: one red.release after the block barrier (publishes the block's
+// partial row) or __threadfence + atomicAdd; tools/fence_probe.py.
+constexpr bool kGridReleaseArrive = true;
+
 __device__ __forceinline__ void grid_barrier(unsigned int *gbar) {
     __syncthreads();
     if (threadIdx.x == 0) {
-        __threadfence();  // publish this block's partial row
-        atomicAdd(gbar, 1u);
+        if constexpr (kGridReleaseArrive) {
+            red_release_add(gbar, 1u);
+        } else {
+            __threadfence();  // publish this block's partial row
+            atomicAdd(gbar, 1u);
+        }
         unsigned int v;
         do {
-            asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(gbar) : "memory");
+            v = ld_acquire_gpu(gbar);
             if (v < gridDim.x) __nanosleep(64);
         } while (v < gridDim.x);
     }

@@ -61,6 +61,25 @@ __device__ __forceinline__ float hsum4(const float4 v) {
     return __fadd_rn(__fadd_rn(v.x, v.y), __fadd_rn(v.z, v.w));
 }
 
+// GPU-scope release / acquire-release counters (PTX memory model).  A block
+// publishes its partial with ONE release operation after a block barrier
+// (cumulativity covers the other threads' stores), instead of
+// __threadfence() + atomicAdd: __threadfence is fence.sc (MEMBAR.SC.GPU plus an
+// L1 invalidate), stronger than the release these hand-offs need.
+__device__ __forceinline__ void red_release_add(unsigned int *p, unsigned int v) {
+    asm volatile("red.release.gpu.global.add.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+__device__ __forceinline__ unsigned int atom_acq_rel_add(unsigned int *p, unsigned int v) {
+    unsigned int r;
+    asm volatile("atom.acq_rel.gpu.global.add.u32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+    return r;
+}
+__device__ __forceinline__ unsigned int ld_acquire_gpu(const unsigned int *p) {
+    unsigned int v;
+    asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+    return v;
+}
+
 // Drop one 128-byte L2 line without writing it back (PTX discard.global.L2).
 // Used on partial-sum rows once their only reader has consumed them: the next
 // launch rewrites them, so their dirty lines would otherwise cost a DRAM

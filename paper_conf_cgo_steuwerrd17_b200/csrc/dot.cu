@@ -19,6 +19,10 @@
 
 namespace lift {
 
+// ticket hand-off: one atom.acq_rel (true) or __threadfence + atomicAdd (false);
+// tools/fence_probe.py
+constexpr bool kDotAcqRelTicket = true;
+
 template <int TPB, int U>
 __device__ __forceinline__ float block_sum(float v, float *red) {
     constexpr int W = TPB / kWarp;
@@ -95,15 +99,22 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
     float bs = block_sum<TPB, U>(s, red);
     if (threadIdx.x == 0) {
         partials[blockIdx.x] = bs;
-        __threadfence();
-        const unsigned int t = atomicAdd(ticket, 1u);
+        // release: publishes this block's partial; acquire: the last block then
+        // sees every other block's (its threads read them after the barrier below)
+        unsigned int t;
+        if constexpr (kDotAcqRelTicket) {
+            t = atom_acq_rel_add(ticket, 1u);
+        } else {
+            __threadfence();
+            t = atomicAdd(ticket, 1u);
+        }
         am_last = (t == gridDim.x - 1);
     }
     __syncthreads();
     if (!am_last) return;
     // second stage (L422-426), fixed order: thread j folds partials j, j+TPB, ...
     // (8 predicated loads in flight, added in that order)
-    __threadfence();
+    if constexpr (!kDotAcqRelTicket) __threadfence();
     float p = 0.f;
     for (int j0 = threadIdx.x; j0 < (int)gridDim.x; j0 += 8 * TPB) {
         float v[8];
