@@ -147,14 +147,22 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
     }
 }
 
+// launch shape (tools/dot_shape_probe.py)
+constexpr int kDotTPB = 256;
+constexpr int kDotU = 4;
+constexpr int kWaves = 2;
+constexpr int64_t kUnitsPerThreadSmall = 2;
+// below this many float4 units one resident wave beats two (profiles/r01w_dot_shape.txt:
+// 2^22 elements 9.95 -> 8.5 us, 2^26 78.3 -> 77.1; at 2^30 two waves stay 0.6 % ahead)
+constexpr int64_t kOneWaveUnits = int64_t(1) << 25;
+
 cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const float *y, float *result,
                        void *workspace, cudaStream_t s, Exch ex) {
     // B200 read sweep (tools/readbw.cu, profiles/r01j_readbw.txt): 256-thread blocks with
     // U = 4 float4 pairs in flight per thread and TWO waves of blocks stream fastest
     // (7.48 TB/s vs 7.39 for 512 threads / one wave); later blocks fill the tail.
-    constexpr int TPB = 256;
-    constexpr int U = 4;
-    constexpr int kWaves = 2;
+    constexpr int TPB = kDotTPB;
+    constexpr int U = kDotU;
     unsigned int *ticket = static_cast<unsigned int *>(workspace);
     float *partials = reinterpret_cast<float *>(static_cast<char *>(workspace) + kDotTicketBytes);
     const bool vec = ((reinterpret_cast<uintptr_t>(x) | reinterpret_cast<uintptr_t>(y)) & 15) == 0;
@@ -168,9 +176,8 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     // small n: two units per thread (both loads in flight in the unrolled tail) and
     // half the blocks of one unit per thread: fewer tickets and partials for the
     // second stage; 2^20: 5.2 us vs 6.7 (profiles/r01s_dot_small.txt)
-    constexpr int64_t kUnitsPerThreadSmall = 2;
     int64_t want = (units + TPB * kUnitsPerThreadSmall - 1) / (TPB * kUnitsPerThreadSmall);
-    int64_t cap = (int64_t)d.sms * per_sm * kWaves;
+    int64_t cap = (int64_t)d.sms * per_sm * (units < kOneWaveUnits ? 1 : kWaves);
     if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;
     int blocks = (int)(want < 1 ? 1 : (want > cap ? cap : want));
     if (vec)
@@ -185,8 +192,8 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
 // spinning on a peer's flag, as the fused collectives do, would never let it).
 cudaError_t preload_dot() {
     cudaFuncAttributes a;
-    cudaError_t e = cudaFuncGetAttributes(&a, k_dot<256, 4, true>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_dot<256, 4, false>);
+    cudaError_t e = cudaFuncGetAttributes(&a, k_dot<kDotTPB, kDotU, true>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_dot<kDotTPB, kDotU, false>);
     return e;
 }
 
