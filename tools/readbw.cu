@@ -128,6 +128,57 @@ __global__ void __launch_bounds__(256, 1) k_bulk(int64_t bytes_per_block, int ch
     if (acc == 12345.f) out[0] = acc;
 }
 
+// ---- bulk-copy dot: x and y streamed as chunk PAIRS into a ring of NST slot
+// pairs (one mbarrier per pair), `bpsm` blocks per SM; chunk j of the grid's
+// sequence goes to block j % G (cyclic: the grid reads one compact window of
+// each array) or block j / per_block (banded).  TPB threads fold x.y from smem.
+template <int TPB>
+__global__ void __launch_bounds__(TPB) k_bulkdot(int64_t nchunks_total, int chunk, int nst, int cyclic,
+                                                 const char *x, const char *y, float *out) {
+    extern __shared__ __align__(128) unsigned char sm[];
+    uint64_t *full = (uint64_t *)sm;
+    char *ring = (char *)(sm + 1024);
+    const int64_t G = gridDim.x, b = blockIdx.x;
+    const int64_t mine = cyclic ? (nchunks_total - b + G - 1) / G : nchunks_total / G;
+    auto src_off = [&](int64_t c) -> int64_t { return (cyclic ? c * G + b : b * mine + c) * (int64_t)chunk; };
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < nst; ++i) asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(su32(full + i)));
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncthreads();
+    auto issue = [&](int64_t c) {
+        const int st = (int)(c % nst);
+        char *dx = ring + (int64_t)st * 2 * chunk;
+        asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(su32(full + st)), "r"(2 * chunk)
+                     : "memory");
+        asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                         su32(dx)), "l"(x + src_off(c)), "r"(chunk), "r"(su32(full + st)) : "memory");
+        asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                         su32(dx + chunk)), "l"(y + src_off(c)), "r"(chunk), "r"(su32(full + st)) : "memory");
+    };
+    if (threadIdx.x == 0)
+        for (int64_t c = 0; c < nst && c < mine; ++c) issue(c);
+    float4 acc = make_float4(0, 0, 0, 0);
+    for (int64_t c = 0; c < mine; ++c) {
+        const int st = (int)(c % nst);
+        const uint32_t ph = (uint32_t)((c / nst) & 1);
+        asm volatile("{\n.reg .pred p;\nW_%=:\nmbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n@!p bra W_%=;\n}\n" ::"r"(
+                         su32(full + st)), "r"(ph) : "memory");
+        const float4 *rx = (const float4 *)(ring + (int64_t)st * 2 * chunk);
+        const float4 *ry = (const float4 *)(ring + (int64_t)st * 2 * chunk + chunk);
+        for (int i = threadIdx.x; i < chunk / 16; i += TPB) {
+            const float4 a = rx[i], bb = ry[i];
+            acc.x = fmaf(a.x, bb.x, acc.x);
+            acc.y = fmaf(a.y, bb.y, acc.y);
+            acc.z = fmaf(a.z, bb.z, acc.z);
+            acc.w = fmaf(a.w, bb.w, acc.w);
+        }
+        __syncthreads();
+        if (threadIdx.x == 0 && c + nst < mine) issue(c + nst);
+    }
+    if (acc.x + acc.y + acc.z + acc.w == 12345.f) out[0] = 1.f;
+}
+
 // fill with non-constant data (zero pages may be served compressed)
 __global__ void k_fill(float *p, int64_t n, uint32_t seed) {
     for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (int64_t)gridDim.x * blockDim.x) {
@@ -175,6 +226,52 @@ int main(int argc, char **argv) {
     k_fill<<<4096, 256>>>(y, n, 2u);
     cudaDeviceSynchronize();
     const float4 *x4 = (const float4 *)x, *y4 = (const float4 *)y;
+    if (argc > 1 && argv[1][0] == 'd') {
+        // bulk-copy dot over x, y (4 GiB each) vs the LDG dot (k4<4,0>, 256 threads, 2 waves)
+        int sms = 0;
+        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
+        auto timeit = [&](auto launch) {
+            cudaEvent_t a, b;
+            cudaEventCreate(&a);
+            cudaEventCreate(&b);
+            float best = 1e30f;
+            for (int it = 0; it < 6; ++it) {
+                cudaEventRecord(a);
+                launch();
+                cudaEventRecord(b);
+                cudaEventSynchronize(b);
+                float ms;
+                cudaEventElapsedTime(&ms, a, b);
+                if (it >= 1 && ms < best) best = ms;
+            }
+            return best;
+        };
+        for (int rep = 0; rep < 2; ++rep) {
+            int per_sm = 0;
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k4<4, 0>, 256, 0);
+            float t = timeit([&] { k4<4, 0><<<per_sm * sms * 2, 256>>>(n / 4, x4, y4, out); });
+            printf("ldg  dot 8 GiB  v4 na U4 256 thr x2 waves                 %9.1f us  %7.1f GB/s\n", t * 1e3,
+                   8.0 * n / (t * 1e-3) / 1e9);
+            for (int bpsm : {1, 2})
+                for (int chunk : {16384, 32768})
+                    for (int nst : {2, 3, 4})
+                        for (int cyc : {0, 1}) {
+                            const size_t smem = 1024 + (size_t)nst * 2 * chunk;
+                            if (smem * bpsm > 225 * 1024) continue;
+                            cudaFuncSetAttribute(k_bulkdot<256>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+                            const int64_t nch = 4 * n / chunk;
+                            const int G = sms * bpsm;
+                            float tb = timeit([&] {
+                                k_bulkdot<256><<<G, 256, smem>>>(nch, chunk, nst, cyc, (const char *)x, (const char *)y, out);
+                            });
+                            printf("bulk dot 8 GiB  %d blk/SM chunk %5d x2  ring %d  %s  %9.1f us  %7.1f GB/s\n", bpsm,
+                                   chunk, nst, cyc ? "cyclic" : "banded", tb * 1e3,
+                                   (double)(cyc ? nch : nch / G * G) * chunk * 2 / (tb * 1e-3) / 1e9);
+                        }
+        }
+        printf("status %s\n", cudaGetErrorString(cudaGetLastError()));
+        return 0;
+    }
     if (argc > 1 && argv[1][0] == 'b') {
         // bulk-copy streaming of 256 MiB / 2 GiB: chunk size x ring depth
         int sms = 0;
