@@ -32,6 +32,15 @@
  *             this changes which rows each block's partial sums, so results
  *             are bitwise those of the untuned call only at the automatic
  *             setting
+ *   cluster   second stage (the sum of the per-block partial rows of y):
+ *             1 = grid barrier of a cooperative launch of one block per SM,
+ *             then every block sums a column slice over all partial rows;
+ *             2, 4, 8 or 16 = thread-block clusters of that size fold their
+ *             partial rows through distributed shared memory into one row
+ *             per cluster, and per column slice the last cluster to arrive
+ *             sums the cluster rows (the grid is the number of such clusters
+ *             that fit at once); 0 = automatic.  Like `cyclic`, this changes
+ *             the summation order: bitwise the untuned call only at 0
  *
  * An unsupported combination returns LIFT_ERR_CUDA with
  * lift_last_cuda_error() = "invalid argument".
@@ -54,6 +63,7 @@ LIFT_API int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *
 
 LIFT_API int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y,
                                    void *workspace, size_t workspace_bytes, int nst, int l2_ahead, int cyclic,
+                                   int cluster,
                                    lift_stream_t stream);
 
 #ifdef __cplusplus

@@ -264,6 +264,13 @@ constexpr int kFusedSmemBudget = 200 * 1024;
 constexpr int kFusedMaxStages = 16;
 constexpr int64_t kFusedMinN = 256;  // below this, rows are too short to stream efficiently
 
+// Cluster form of the fused kernel's second stage (kernel argument clu):
+// cluster sizes up to kFusedMaxCluster; per-slice arrival tickets live in the
+// workspace header at gbar[kClusterTicket + r] (zero before first use, re-armed
+// by the last arrival).
+constexpr int kFusedMaxCluster = 16;
+constexpr int kClusterTicket = 16;
+
 struct FusedPlan {
     int qc;       // float4 columns per thread (1, 2, 4, 8)
     int cr;       // rows per step
@@ -272,6 +279,7 @@ struct FusedPlan {
     int cyc;      // 1: stages assigned to blocks cyclically, 0: contiguous bands
     size_t hdr;   // barrier + reduction header bytes
     size_t smem;  // dynamic smem bytes
+    int clu;      // second stage: cluster size (0 = grid barrier)
 };
 
 // Stage = CR consecutive rows moved by ONE bulk copy; each consumer step takes
@@ -284,7 +292,14 @@ constexpr size_t kFusedStageTarget = 32 * 1024;
 constexpr size_t kFusedRingTarget = 112 * 1024;
 constexpr int kFusedL2Ahead = 0;
 constexpr int kFusedCyclic = 1;
-constexpr int kFusedXsmemQc = 8;  // qc at which x moves from registers to shared memory
+constexpr int kFusedXsmemQc = 8;
+// Second stage by default: the grid barrier (0).  Clusters of C blocks folding
+// their partial rows through DSMEM (tuning option cluster = C) measured slower
+// at every shape (profiles/r01y_atax_cluster_probe.txt): one block per SM packs
+// into fewer SMs as clusters (C = 4 / 8 / 16: 132 / 120 / 112 blocks, and the
+// ring stream needs every SM), and with C = 2 (148 blocks) the last cluster's
+// sum over 74 cluster rows is one serial chain.
+constexpr int kFusedCluster = 0;  // qc at which x moves from registers to shared memory
 
 static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}) {
     if (n <= 0 || n % 4 != 0) return false;
@@ -317,9 +332,15 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
     p->l2a = tune.l2a >= 0 ? tune.l2a : kFusedL2Ahead;
     p->cyc = tune.cyc >= 0 ? tune.cyc : kFusedCyclic;
     p->hdr = hdr;
-    // the drained ring is reused for the final column-sum tile partials
+    if (tune.clu < 0 || tune.clu > kFusedMaxCluster || (tune.clu & (tune.clu - 1)) != 0) return false;
+    p->clu = tune.clu == 0 ? kFusedCluster : (tune.clu == 1 ? 0 : tune.clu);
+    // the drained ring is reused for the final column-sum tile partials (grid-barrier
+    // form) or for this block's partial row and one float4 per thread (cluster form)
     const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
-    p->smem = hdr + (ring > tile ? ring : tile) + xs_bytes;
+    const size_t crow = (size_t)(n + 31) / 32 * 128 + (size_t)kFusedThreads * 16;
+    size_t tail = ring > tile ? ring : tile;
+    if (p->clu > 0 && crow > tail) tail = crow;
+    p->smem = hdr + tail + xs_bytes;
     return true;
 }
 
@@ -393,6 +414,60 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
     }
 }
 
+
+// y[c] = sum_{k < K} P[k][c] for the vector columns c in [c0, c1), by one
+// block, in a fixed order: each pass covers cw = T/g columns with g row
+// groups (contiguous, in order; 8 loads in flight per thread), then the g
+// group sums of a column are added in group order.  The order depends only
+// on (K, c1 - c0).
+__device__ __forceinline__ void colsum_rows(int K, int64_t nv, const float4 *__restrict__ P4,
+                                           float4 *__restrict__ y4, int64_t c0, int64_t c1,
+                                           float4 *part /* smem [kFusedThreads] */) {
+    const int tid = threadIdx.x;
+    const int64_t w = c1 - c0;
+    if (w <= 0) return;
+    int g = w >= kFusedThreads ? 1 : (int)(kFusedThreads / w);
+    if (g > K) g = K;
+    const int cw = kFusedThreads / g;
+    const int col = tid % cw, grp = tid / cw;
+    const int k0 = grp < g ? K * grp / g : 0, k1 = grp < g ? K * (grp + 1) / g : 0;
+    for (int64_t cb = c0; cb < c1; cb += cw) {
+        const int64_t c = cb + col;
+        float4 acc = zero4();
+        if (c < c1) {
+            for (int k = k0; k < k1; k += 8) {
+                float4 v[8];
+#pragma unroll
+                for (int u = 0; u < 8; ++u)
+                    if (k + u < k1) v[u] = __ldcg(P4 + (int64_t)(k + u) * nv + c);
+#pragma unroll
+                for (int u = 0; u < 8; ++u) {
+                    if (k + u < k1) {
+                        acc.x = __fadd_rn(acc.x, v[u].x);
+                        acc.y = __fadd_rn(acc.y, v[u].y);
+                        acc.z = __fadd_rn(acc.z, v[u].z);
+                        acc.w = __fadd_rn(acc.w, v[u].w);
+                    }
+                }
+            }
+        }
+        part[tid] = acc;
+        __syncthreads();
+        if (tid < cw && c < c1) {
+            float4 s = part[tid];
+            for (int j = 1; j < g; ++j) {
+                const float4 v = part[j * cw + tid];
+                s.x = __fadd_rn(s.x, v.x);
+                s.y = __fadd_rn(s.y, v.y);
+                s.z = __fadd_rn(s.z, v.z);
+                s.w = __fadd_rn(s.w, v.w);
+            }
+            y4[c] = s;
+        }
+        __syncthreads();
+    }
+}
+
 // The fused kernel's partial rows may be discarded from L2 after their last
 // read only when every row is a whole number of 128-byte lines (no line shared
 // by two rows).  Measured (profiles/r01u_atax_discard.txt): fused ATAX 8192^2
@@ -441,7 +516,7 @@ template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
     k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
                  float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar, Exch ex,
-                 int dst, int l2a, int cyc, bool discard_partials) {
+                 int dst, int l2a, int cyc, bool discard_partials, int clu) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
@@ -595,6 +670,54 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
             phase ^= 1u;
         }
     }
+    if (clu) {
+        // ---- second stage, cluster form: the C blocks of a cluster fold their
+        // partial y rows through distributed shared memory into ONE row per
+        // cluster (block r owns vector-column slice r), then per slice the last
+        // of the K clusters to publish it sums the K cluster rows.  No grid
+        // barrier, no cooperative launch; the order is fixed by (n, C, K). ----
+        float4 *row4 = reinterpret_cast<float4 *>(stage0);  // the drained ring
+#pragma unroll
+        for (int q = 0; q < QC; ++q) {
+            const int64_t c = tid + (int64_t)kFusedThreads * q;
+            if (c < nv) row4[c] = yr[q];
+        }
+        cluster_sync();  // every block's row is in its smem
+        const uint32_t C = cluster_nctarank(), r = cluster_ctarank();
+        const int K = (int)cluster_count_x();
+        const int64_t cid = cluster_id_x();
+        const int64_t c0 = nv * r / C, c1 = nv * (r + 1) / C;
+        float4 *P4 = reinterpret_cast<float4 *>(P);
+        for (int64_t c = c0 + tid; c < c1; c += kFusedThreads) {
+            float4 v[kFusedMaxCluster];
+            const uint32_t la = smem_u32(row4 + c);
+#pragma unroll
+            for (int b = 0; b < kFusedMaxCluster; ++b)
+                if (b < (int)C) v[b] = ld_dsmem4(dsmem_addr_raw(la, b));
+            float4 acc = v[0];
+#pragma unroll
+            for (int b = 1; b < kFusedMaxCluster; ++b) {
+                if (b < (int)C) {
+                    acc.x = __fadd_rn(acc.x, v[b].x);
+                    acc.y = __fadd_rn(acc.y, v[b].y);
+                    acc.z = __fadd_rn(acc.z, v[b].z);
+                    acc.w = __fadd_rn(acc.w, v[b].w);
+                }
+            }
+            __stcg(P4 + cid * nv + c, acc);
+        }
+        cluster_arrive();  // this block's DSMEM reads are done (waited for before exit)
+        __shared__ int is_last;
+        __syncthreads();   // the slice of this cluster's row is written
+        if (tid == 0) is_last = atom_acq_rel_add(gbar + kClusterTicket + r, 1u) == (unsigned)(K - 1);
+        __syncthreads();
+        if (is_last) {
+            colsum_rows(K, nv, P4, reinterpret_cast<float4 *>(y), c0, c1, row4 + (nv + 7) / 8 * 8);
+            if (tid == 0) gbar[kClusterTicket + r] = 0u;  // every cluster has arrived: re-arm
+        }
+        cluster_wait();  // no block leaves while a peer may still read its smem
+        return;
+    }
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
 #pragma unroll
     for (int q = 0; q < QC; ++q) {
@@ -657,25 +780,78 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 }
 
 template <int QC, int CR>
-static cudaError_t run_fused(const FusedPlan &p, int64_t m, int64_t n, const float *A, const float *x, float *P,
-                             float *y, unsigned int *gbar, int blocks, cudaStream_t s, const Exch &ex, int dst,
-                             bool cooperative) {
-    auto k = k_atax_fused<QC, CR>;
-    cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
-    if (e != cudaSuccess) return e;
-    // cooperative: the in-kernel grid barrier needs every block resident (one per SM)
+static cudaLaunchConfig_t fused_cfg(const FusedPlan &p, int blocks, int clu, bool cooperative, cudaStream_t s,
+                                    cudaLaunchAttribute *attr) {
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3((unsigned)blocks);
     cfg.blockDim = dim3(kFusedThreads);
     cfg.dynamicSmemBytes = p.smem;
     cfg.stream = s;
-    cudaLaunchAttribute attr[1];
-    attr[0].id = cudaLaunchAttributeCooperative;
-    attr[0].val.cooperative = 1;
     cfg.attrs = attr;
-    cfg.numAttrs = cooperative ? 1 : 0;
+    cfg.numAttrs = 0;
+    if (clu > 0) {  // cluster form: no grid barrier, no co-residency needed
+        attr[0].id = cudaLaunchAttributeClusterDimension;
+        attr[0].val.clusterDim.x = (unsigned)clu;
+        attr[0].val.clusterDim.y = 1;
+        attr[0].val.clusterDim.z = 1;
+        cfg.numAttrs = 1;
+    } else if (cooperative) {  // the in-kernel grid barrier needs every block resident (one per SM)
+        attr[0].id = cudaLaunchAttributeCooperative;
+        attr[0].val.cooperative = 1;
+        cfg.numAttrs = 1;
+    }
+    return cfg;
+}
+
+// Clusters of `clu` blocks (one per SM) that fit at once for this plan, cached
+// per (device, kernel shape, smem, clu); 0 if the cluster shape cannot launch.
+template <int QC, int CR>
+static int fused_max_clusters(const DeviceInfo &d, const FusedPlan &p, int clu) {
+    struct Entry {
+        int dev, nst, clu;
+        size_t smem;
+        int k;
+    };
+    static Entry cache[32];
+    static int used = 0;
+    for (int i = 0; i < used; ++i)
+        if (cache[i].dev == d.device && cache[i].nst == p.nst && cache[i].clu == clu && cache[i].smem == p.smem)
+            return cache[i].k;
+    auto k = k_atax_fused<QC, CR>;
+    cudaLaunchAttribute attr[1];
+    cudaLaunchConfig_t cfg = fused_cfg<QC, CR>(p, clu * (d.sms / clu), clu, false, 0, attr);
+    int nc = 0;
+    if (cudaOccupancyMaxActiveClusters(&nc, k, &cfg) != cudaSuccess) {
+        (void)cudaGetLastError();
+        nc = 0;
+    }
+    if (used < 32) cache[used++] = Entry{d.device, p.nst, clu, p.smem, nc};
+    return nc;
+}
+
+template <int QC, int CR>
+static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m, int64_t n, const float *A,
+                             const float *x, float *P, float *y, unsigned int *gbar, int blocks, cudaStream_t s,
+                             const Exch &ex, int dst, bool cooperative, int clu) {
+    auto k = k_atax_fused<QC, CR>;
+    cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
+    if (e != cudaSuccess) return e;
+    if (clu > 0) {
+        if (clu > 8) {
+            e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+            if (e != cudaSuccess) return e;
+        }
+        int64_t K = fused_max_clusters<QC, CR>(d, p, clu);
+        if (K < 1) return cudaErrorInvalidConfiguration;
+        if (K * clu > kMaxSplits) K = kMaxSplits / clu;
+        const int64_t need = (m + clu - 1) / clu;  // at least one row per cluster
+        if (K > need) K = need < 1 ? 1 : need;
+        blocks = (int)(K * clu);
+    }
+    cudaLaunchAttribute attr[1];
+    cudaLaunchConfig_t cfg = fused_cfg<QC, CR>(p, blocks, clu, cooperative, s, attr);
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.l2a, p.cyc,
-                              rows_are_lines(P, n));
+                              rows_are_lines(P, n), clu);
 }
 
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)
@@ -710,9 +886,13 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     // block count (tests running several ranks on one GPU) launches plainly
     const bool cooperative = blocks <= 0;
     if (blocks > 0) G = blocks < G ? blocks : G;
+    // second stage: clusters of p.clu blocks (single rank, grid chosen from the
+    // cluster occupancy), else the grid barrier (exchanges, explicit grids)
+    const int clu = (ex.world == 0 && blocks <= 0 && m > 0) ? p.clu : 0;
     cudaError_t e = cudaErrorInvalidValue;
-#define LIFT_FUSED_CASE(QC, CR) \
-    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(p, m, n, A, x, P, y, gbar, (int)G, s, ex, dst, cooperative);
+#define LIFT_FUSED_CASE(QC, CR)                                                                                     \
+    if (p.qc == QC && p.cr == CR)                                                                                   \
+        e = run_fused<QC, CR>(d, p, m, n, A, x, P, y, gbar, (int)G, s, ex, dst, cooperative, clu);
     // fused_plan pairs: qc 1 -> cr 4 (rows <= 8 KiB), qc 2 -> cr 2, qc 4 / 8 -> cr 1
     LIFT_FUSED_CASE(1, 4)
     LIFT_FUSED_CASE(1, 2)

@@ -352,6 +352,32 @@ def test_atax_fused_tuning(cuda_device):
                 lift.lift_atax_fused_tuned(A, x, **bad)
 
 
+@pytest.mark.parametrize("cluster", [1, 2, 4, 8, 16])
+def test_atax_fused_cluster(cuda_device, cluster):
+    """lift_atax_fused_tuned(cluster=C): the second stage (sum of the
+    per-block partial rows of y) by the grid barrier (C = 1) or by clusters
+    of C blocks folding their rows through distributed shared memory, then
+    the last cluster per column slice summing the cluster rows.  Every form
+    meets the oracle's tolerance, repeats bitwise (the per-slice tickets
+    re-arm), and is rejected for sizes that are not a power of two <= 16."""
+    shapes = ((1, 256), (3, 8192), (15, 1028), (1000, 4096), (777, 8192), (300, 16384), (5000, 516), (4096, 4096))
+    for m, n in shapes:
+        A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+        x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+        ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+        got = lift.lift_atax_fused_tuned(A, x, cluster=cluster)
+        assert_tol(got.cpu().numpy(), ref, mag, f"atax cluster {cluster} {m}x{n}")
+        for _ in range(3):
+            assert torch.equal(lift.lift_atax_fused_tuned(A, x, cluster=cluster), got), (m, n, cluster)
+        if cluster == 1:  # the automatic second stage is the grid barrier
+            assert torch.equal(lift.lift_atax(A, x, algo="fused"), got), (m, n)
+    A = synth.torch_matrix_rows(synth.SEED_A, 512, 0, 64, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, 512, device=cuda_device)
+    for bad in (3, 32, -1):
+        with pytest.raises(lift.LiftError):
+            lift.lift_atax_fused_tuned(A, x, cluster=bad)
+
+
 @pytest.mark.parametrize("algo", ["fused", "twopass"])
 def test_atax_full_size_8192(cuda_device, algo):
     """configs[3] at one GPU, every output."""
