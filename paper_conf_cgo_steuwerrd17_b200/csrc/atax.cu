@@ -468,6 +468,55 @@ __device__ __forceinline__ void colsum_rows(int K, int64_t nv, const float4 *__r
     }
 }
 
+// In-warp sums of CR row partials d[0..CR) (one per lane each), as CR
+// butterflies xor 16, 8, 4, 2, 1 would give them, with the first log2(CR)
+// levels folded: at level xor 16 (CR >= 2) the lower half-warp keeps rows
+// [0, CR/2) and the upper half rows [CR/2, CR), each lane sending its partner
+// the rows the partner keeps; at xor 8 (CR = 4) the same within each half.
+// Every add pairs the same two partial sums as the plain butterfly (fp add is
+// commutative), so the bits are those of CR separate butterflies.  Returns
+// this lane's value; row i's sum is in lanes [i*32/CR, (i+1)*32/CR).
+template <int CR>
+__device__ __forceinline__ float row_butterfly(const float (&d)[CR], int lane) {
+    float v;
+    if constexpr (CR == 1) {
+        v = d[0];
+    } else if constexpr (CR == 2) {
+        const bool hi = lane & 16;
+        v = __fadd_rn(hi ? d[1] : d[0], __shfl_xor_sync(0xffffffffu, hi ? d[0] : d[1], 16));
+    } else {
+        static_assert(CR == 4, "CR is 1, 2 or 4");
+        const bool hi = lane & 16;
+        const float k0 = __fadd_rn(hi ? d[2] : d[0], __shfl_xor_sync(0xffffffffu, hi ? d[0] : d[2], 16));
+        const float k1 = __fadd_rn(hi ? d[3] : d[1], __shfl_xor_sync(0xffffffffu, hi ? d[1] : d[3], 16));
+        const bool h8 = lane & 8;
+        v = __fadd_rn(h8 ? k1 : k0, __shfl_xor_sync(0xffffffffu, h8 ? k0 : k1, 8));
+    }
+#pragma unroll
+    for (int o = 16 / CR; o > 0; o >>= 1) v = __fadd_rn(v, __shfl_xor_sync(0xffffffffu, v, o));
+    return v;
+}
+
+// t[i] = pair_tree over the kFusedWarps = 16 warp sums pb[i*16 .. i*16+15]
+// for i < CR, in every lane: each half-warp loads one row's 16 sums and runs
+// the butterfly xor 1, 2, 4, 8, which adds exactly the pairs of the pairwise
+// tree level by level (same bits as pair_tree<16>), then lane 0 / 16
+// broadcasts.  Two rows per pass instead of 4 vector loads + 15 adds per row
+// in every thread.
+template <int CR>
+__device__ __forceinline__ void warp_trees(const float *pb, int lane, float (&t)[CR]) {
+    static_assert(kFusedWarps == 16, "one half-warp per row of warp sums");
+#pragma unroll
+    for (int i0 = 0; i0 < CR; i0 += 2) {
+        const int row = (CR == 1) ? 0 : i0 + (lane >> 4);
+        float v = pb[row * kFusedWarps + (lane & 15)];
+#pragma unroll
+        for (int o = 1; o < 16; o <<= 1) v = __fadd_rn(v, __shfl_xor_sync(0xffffffffu, v, o));
+        t[i0] = __shfl_sync(0xffffffffu, v, 0);
+        if (i0 + 1 < CR) t[i0 + 1] = __shfl_sync(0xffffffffu, v, 16);
+    }
+}
+
 // The fused kernel's partial rows may be discarded from L2 after their last
 // read only when every row is a whole number of 128-byte lines (no line shared
 // by two rows).  Measured (profiles/r01u_atax_discard.txt): fused ATAX 8192^2
@@ -586,19 +635,18 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     int slot = 0;        // ring slot of stage k (k % nst), tracked without division
     uint32_t phase = 0;  // its mbarrier phase parity ((k / nst) & 1)
     int pslot = 0;       // ring slot of stage k-1
-    float4 ap[CR][QC];   // the previous stage's rows, kept for its rank-1 updates
-#pragma unroll
-    for (int i = 0; i < CR; ++i)
-#pragma unroll
-        for (int q = 0; q < QC; ++q) ap[i][q] = zero4();
-    for (int64_t k = 0;; ++k, buf ^= 1) {
+    int64_t k = 0;
+    // Two register sets of CR rows: one step loads the current stage into `cur`
+    // and applies the previous stage's updates from `prev`; steps alternate the
+    // roles (no register copies between steps).  Returns true after the last.
+    float4 ra[CR][QC], rb2[CR][QC];
+    auto step = [&](float4(&cur)[CR][QC], float4(&prev)[CR][QC]) -> bool {
         const int rows = stage_rows(k);
         __syncthreads();  // previous stage: partials published, slot consumed
         if (tid == 0 && prow > 0 && k - 1 + nst < nstages) {
             issue_stage(k - 1 + nst, pslot);
             if (l2a > 0) prefetch_stage(k - 1 + nst + l2a);
         }
-        float4 a[CR][QC];
         float *rb = red + buf * CR * kFusedWarps;
         if (rows > 0) {
             mbar_wait_parity(full + slot, phase);
@@ -608,7 +656,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 #pragma unroll
                 for (int q = 0; q < QC; ++q) {
                     const int64_t c = tid + (int64_t)kFusedThreads * q;
-                    a[i][q] = (i < rows && c < nv) ? S4[(int64_t)i * nv + c] : zero4();
+                    cur[i][q] = (i < rows && c < nv) ? S4[(int64_t)i * nv + c] : zero4();
                 }
             }
             // partial dots of this thread's columns, CR rows at once
@@ -620,55 +668,46 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
                 for (int q = 0; q < QC; ++q) {
                     if constexpr (XS) {
                         const int64_t c = tid + (int64_t)kFusedThreads * q;
-                        fma4(acc, a[i][q], c < nv ? xs4[c] : zero4());
+                        fma4(acc, cur[i][q], c < nv ? xs4[c] : zero4());
                     } else {
-                        fma4(acc, a[i][q], xr[q]);
+                        fma4(acc, cur[i][q], xr[q]);
                     }
                 }
                 d[i] = hsum4(acc);
             }
-#pragma unroll
-            for (int o = 16; o > 0; o >>= 1)
-#pragma unroll
-                for (int i = 0; i < CR; ++i) d[i] = __fadd_rn(d[i], __shfl_xor_sync(0xffffffffu, d[i], o));
-            if (lane == 0) {
-#pragma unroll
-                for (int i = 0; i < CR; ++i) rb[i * kFusedWarps + warp] = d[i];
-            }
+            // warp butterflies of the CR rows, folded so each level moves one value
+            // per lane: row i's sum ends in lane i * 32 / CR (same bits as CR
+            // separate butterflies, row_butterfly)
+            const float dr = row_butterfly<CR>(d, lane);
+            if ((lane & (32 / CR - 1)) == 0) rb[(lane / (32 / CR)) * kFusedWarps + warp] = dr;
         }
         // rank-1 updates of the previous stage: y += A_r^T t_r
         if (prow > 0) {
             const float *pb = red + (buf ^ 1) * CR * kFusedWarps;
+            float t[CR];  // t_r = A_r . x: the pairwise tree over the 16 warp sums
+            warp_trees<CR>(pb, lane, t);
 #pragma unroll
             for (int i = 0; i < CR; ++i) {
                 if (i < prow) {
-                    float v[kFusedWarps];
-                    const float4 *rb4 = reinterpret_cast<const float4 *>(pb + i * kFusedWarps);
 #pragma unroll
-                    for (int w = 0; w < kFusedWarps / 4; ++w) {
-                        const float4 t4 = rb4[w];
-                        v[4 * w] = t4.x;
-                        v[4 * w + 1] = t4.y;
-                        v[4 * w + 2] = t4.z;
-                        v[4 * w + 3] = t4.w;
-                    }
-                    const float t = pair_tree<kFusedWarps>(v);  // t_r = A_r . x
-#pragma unroll
-                    for (int q = 0; q < QC; ++q) fma4s(yr[q], ap[i][q], t);
+                    for (int q = 0; q < QC; ++q) fma4s(yr[q], prev[i][q], t[i]);
                 }
             }
         }
-        if (rows == 0) break;
-#pragma unroll
-        for (int i = 0; i < CR; ++i)
-#pragma unroll
-            for (int q = 0; q < QC; ++q) ap[i][q] = a[i][q];
+        if (rows == 0) return true;
         prow = rows;
         pslot = slot;
         if (++slot == nst) {
             slot = 0;
             phase ^= 1u;
         }
+        ++k;
+        buf ^= 1;
+        return false;
+    };
+    for (;;) {
+        if (step(ra, rb2)) break;
+        if (step(rb2, ra)) break;
     }
     if (clu) {
         // ---- second stage, cluster form: the C blocks of a cluster fold their

@@ -1,0 +1,61 @@
+"""Fused-ATAX launch-shape variants (tuning aid; the library is not changed).
+
+Each variant is a copy of the package under /tmp with textual patches to
+csrc/atax.cu, built and timed by tools/ab_atax.py (bitwise outputs saved, so
+the variants that keep the summation order can be checked against the
+library).  usage: python tools/atax_variant_probe.py [name ...]
+"""
+import os
+import shutil
+import subprocess
+import sys
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+SRC = os.path.join(ROOT, "paper_conf_cgo_steuwerrd17_b200", "csrc", "atax.cu")
+
+CASES = ("    LIFT_FUSED_CASE(1, 4)\n", "    LIFT_FUSED_CASE(1, 4)\n    LIFT_FUSED_CASE(2, 4)\n")
+VARIANTS = {
+    "lib": [],
+    # QC = 2 (n in (2048, 4096]) with 4 rows per step: one barrier per 64 KiB stage
+    "qc2cr4": [("const int cr_max = qc == 1 ? 4 : (qc == 2 ? 2 : 1);", "const int cr_max = qc <= 2 ? 4 : 1;"),
+               ("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 64 * 1024;"),
+               ("constexpr size_t kFusedRingTarget = 112 * 1024;", "constexpr size_t kFusedRingTarget = 128 * 1024;"),
+               CASES],
+    # deeper ring (more bytes in flight per SM)
+    "ring160": [("constexpr size_t kFusedRingTarget = 112 * 1024;", "constexpr size_t kFusedRingTarget = 160 * 1024;")],
+    # 16 KiB stages (more, smaller bulk copies; twice the steps)
+    "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
+}
+
+
+def patched(name):
+    d = f"/tmp/atax_var_{name}"
+    shutil.rmtree(d, ignore_errors=True)
+    os.makedirs(d)
+    for sub in ("paper_conf_cgo_steuwerrd17_b200", "include", "synth", "oracle", "tools"):
+        shutil.copytree(os.path.join(ROOT, sub), os.path.join(d, sub),
+                        ignore=shutil.ignore_patterns("_build", "*.so", "__pycache__"))
+    shutil.copy(os.path.join(ROOT, "__graft_entry__.py"), d)
+    src = open(SRC).read()
+    for old, new in VARIANTS[name]:
+        assert old in src, (name, old)
+        src = src.replace(old, new)
+    open(os.path.join(d, "paper_conf_cgo_steuwerrd17_b200", "csrc", "atax.cu"), "w").write(src)
+    subprocess.run([sys.executable, "-c", "import __graft_entry__ as g; g.build()"], cwd=d, check=True)
+    return d
+
+
+names = sys.argv[1:] or list(VARIANTS)
+res = {}
+for name in names:
+    d = patched(name)
+    print(f"== {name}", flush=True)
+    out = os.path.join(d, "out.npz")
+    subprocess.run([sys.executable, os.path.join(ROOT, "tools", "ab_atax.py"), out], cwd=d, check=True)
+    res[name] = np.load(out)
+if "lib" in res:
+    for name, r in res.items():
+        same = [k for k in r.files if k.startswith("y_") and np.array_equal(r[k], res["lib"][k])]
+        print(name, "bitwise equal to lib at:", ", ".join(s[2:] for s in same))
