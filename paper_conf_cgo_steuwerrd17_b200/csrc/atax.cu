@@ -26,6 +26,7 @@
 // The per-block y partials are summed in a fixed order in the SAME launch: a
 // grid barrier (cooperative launch, one block per SM) and then every block
 // reduces a tile of columns over all partial rows.
+#include <mutex>
 #include <type_traits>
 
 #include "common.cuh"
@@ -853,6 +854,8 @@ static int fused_max_clusters(const DeviceInfo &d, const FusedPlan &p, int clu) 
     };
     static Entry cache[32];
     static int used = 0;
+    static std::mutex mu;  // host threads may launch concurrently
+    std::lock_guard<std::mutex> lock(mu);
     for (int i = 0; i < used; ++i)
         if (cache[i].dev == d.device && cache[i].nst == p.nst && cache[i].clu == clu && cache[i].smem == p.smem)
             return cache[i].k;
