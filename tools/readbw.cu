@@ -60,6 +60,35 @@ __global__ void k4(int64_t n4, const float4 *x, const float4 *y, float *out) {
     if (s == 12345.f) out[0] = s;  // keep the loads alive
 }
 
+// warp-contiguous chunks: warp w streams chunks w, w + W, ... of U*512 bytes per
+// array (its U loads per array are adjacent 512-byte segments: DRAM page locality)
+template <int U>
+__global__ void k4c(int64_t n4, const float4 *x, const float4 *y, float *out) {
+    const int lane = threadIdx.x & 31;
+    const int64_t nw = (int64_t)gridDim.x * blockDim.x / 32;
+    float4 acc[U];
+    for (int u = 0; u < U; ++u) acc[u] = make_float4(0, 0, 0, 0);
+    for (int64_t c = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) / 32; (c + 1) * U * 32 <= n4; c += nw) {
+        const int64_t b = c * U * 32 + lane;
+        float4 a[U], bb[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            a[u] = ld4_na(x + b + u * 32);
+            bb[u] = ld4_na(y + b + u * 32);
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            acc[u].x = fmaf(a[u].x, bb[u].x, acc[u].x);
+            acc[u].y = fmaf(a[u].y, bb[u].y, acc[u].y);
+            acc[u].z = fmaf(a[u].z, bb[u].z, acc[u].z);
+            acc[u].w = fmaf(a[u].w, bb[u].w, acc[u].w);
+        }
+    }
+    float s = 0;
+    for (int u = 0; u < U; ++u) s += acc[u].x + acc[u].y + acc[u].z + acc[u].w;
+    if (s == 12345.f) out[0] = s;
+}
+
 template <int U, int MODE>
 __global__ void k8(int64_t n8, const float *x, const float *y, float *out) {
     const int64_t stride = (int64_t)gridDim.x * blockDim.x;
@@ -226,6 +255,20 @@ int main(int argc, char **argv) {
     k_fill<<<4096, 256>>>(y, n, 2u);
     cudaDeviceSynchronize();
     const float4 *x4 = (const float4 *)x, *y4 = (const float4 *)y;
+    if (argc > 1 && argv[1][0] == 'c') {
+        // grid-strided (k4) vs warp-contiguous chunks (k4c), and one 8 GiB stream vs two 4 GiB streams
+        for (int rep = 0; rep < 2; ++rep) {
+            run("v4 na U4 strided", k4<4, 0>, 256, 8 * n, n / 4, x4, y4, out);
+            run("v4 na U4 warp-chunk 2 KiB", k4c<4>, 256, 8 * n, n / 4, x4, y4, out);
+            run("v4 na U8 warp-chunk 4 KiB", k4c<8>, 256, 8 * n, n / 4, x4, y4, out);
+            run("v4 na U2 warp-chunk 1 KiB", k4c<2>, 256, 8 * n, n / 4, x4, y4, out);
+            // one stream: both operands from x (first and second half): 4 GiB read
+            run("v4 na U4 strided, x halves", k4<4, 0>, 256, 4 * n, n / 8, x4, x4 + n / 8, out);
+            run("v4 na U4 same-array 1 stream", k4<4, 0>, 256, 4 * n, n / 8, x4, x4, out);
+        }
+        printf("status %s\n", cudaGetErrorString(cudaGetLastError()));
+        return 0;
+    }
     if (argc > 1 && argv[1][0] == 'd') {
         // bulk-copy dot over x, y (4 GiB each) vs the LDG dot (k4<4,0>, 256 threads, 2 waves)
         int sms = 0;
