@@ -190,6 +190,29 @@ def test_gemv_nan_propagates(cuda_device):
     assert torch.isnan(lift.lift_gemv(A, x)).all()
 
 
+def test_nan_propagates_every_op(cuda_device):
+    """Reading A14: IEEE propagation, no special-casing — a NaN
+    input element reaches every output that depends on it, in every op and
+    algorithm; outputs that do not depend on it stay finite."""
+    m, n = 300, 1024
+    A = dev_np(rand(2, (m, n)), cuda_device)
+    B = dev_np(rand(3, (m, n)), cuda_device)
+    x = dev_np(rand(0, (n,)), cuda_device)
+    xn = x.clone()
+    xn[517] = float("nan")
+    assert torch.isnan(lift.lift_dot(xn, x)).item()
+    assert torch.isnan(lift.lift_gesummv(1.5, A, 1.2, B, xn)).all()
+    for algo in ("fused", "twopass"):
+        assert torch.isnan(lift.lift_atax(A, xn, algo=algo)).all()  # t is all NaN, so is every y_j
+    # a NaN in one row of A: only that row of A x, but (through t) every y_j of ATAX
+    An = A.clone()
+    An[123, 45] = float("nan")
+    y = lift.lift_gemv(An, x)
+    assert torch.isnan(y[123]) and torch.isfinite(torch.cat([y[:123], y[124:]])).all()
+    for algo in ("fused", "twopass"):
+        assert torch.isnan(lift.lift_atax(An, x, algo=algo)).all()
+
+
 def test_gemv_nondefault_stream_and_graph(cuda_device):
     m, n = 2048, 4096
     A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
