@@ -11,6 +11,7 @@ Sharded (multi-GPU) variants live in :mod:`paper_conf_cgo_steuwerrd17_b200.shard
 """
 from __future__ import annotations
 
+import contextlib
 import threading
 
 import torch
@@ -51,7 +52,23 @@ def _same_device(*ts: torch.Tensor) -> torch.device:
     return d
 
 
+_NULL_CTX = contextlib.nullcontext()
+
+
+def _on(device: torch.device):
+    """torch.cuda.device(device), skipped when it is already current (the
+    common case: switching devices costs a few microseconds per call)."""
+    return _NULL_CTX if device.index == torch.cuda.current_device() else torch.cuda.device(device)
+
+
+# the raw handle of the current stream without building a torch.cuda.Stream
+# object (0.07 instead of 2.2 us per call, tools/binding_profile.py)
+_raw_stream = getattr(torch._C, "_cuda_getCurrentRawStream", None)
+
+
 def _stream(device: torch.device) -> int:
+    if _raw_stream is not None:
+        return _raw_stream(device.index)
     return torch.cuda.current_stream(device).cuda_stream
 
 
@@ -97,7 +114,7 @@ def lift_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None = None) 
     L = lib()
     n = x.numel()
     nbytes = L.lift_dot_workspace_bytes(n)
-    with torch.cuda.device(dev):
+    with _on(dev):
         ws = _workspace("dot", dev, nbytes, zero=True)
         check(L.lift_dot(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(), _stream(dev)))
     return out
@@ -114,7 +131,7 @@ def lift_gemv(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None)
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
-    with torch.cuda.device(dev):
+    with _on(dev):
         check(lib().lift_gemv(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), _stream(dev)))
     return out
 
@@ -127,7 +144,7 @@ def lift_gemv_tuned(A, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1, lb=0):
     m, n = A.shape
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
-    with torch.cuda.device(dev):
+    with _on(dev):
         check(lib().lift_gemv_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), wpr, rg, blocks, xsmem, lb,
                                     _stream(dev)))
     return out
@@ -146,7 +163,7 @@ def lift_gesummv(alpha: float, A: torch.Tensor, beta: float, B: torch.Tensor, x:
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
-    with torch.cuda.device(dev):
+    with _on(dev):
         check(lib().lift_gesummv(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
                                  out.data_ptr(), _stream(dev)))
     return out
@@ -160,7 +177,7 @@ def lift_gesummv_tuned(alpha, A, beta, B, x, out=None, wpr=0, rg=0, blocks=0, xs
     m, n = A.shape
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
-    with torch.cuda.device(dev):
+    with _on(dev):
         check(lib().lift_gesummv_tuned(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
                                        out.data_ptr(), wpr, rg, blocks, xsmem, lb, _stream(dev)))
     return out
@@ -182,7 +199,7 @@ def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None,
     _check_tensor(out, "out", 1)
     L = lib()
     nbytes = L.lift_atax_workspace_bytes(m, n)
-    with torch.cuda.device(dev):
+    with _on(dev):
         ws = _workspace("atax", dev, nbytes, zero=True)
         check(L.lift_atax_algo_run(_ALGOS[algo], m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(),
                                    ws.numel(), _stream(dev)))
@@ -203,7 +220,7 @@ def lift_atax_fused_tuned(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | 
     _check_tensor(out, "out", 1)
     L = lib()
     nbytes = L.lift_atax_workspace_bytes(m, n)
-    with torch.cuda.device(dev):
+    with _on(dev):
         ws = _workspace("atax", dev, nbytes, zero=True)
         check(L.lift_atax_fused_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
                                       nst, l2_ahead, cyclic, cluster, _stream(dev)))
@@ -222,7 +239,7 @@ def lift_partial_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None 
     if out is None:
         out = torch.empty(n // 128, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
-    with torch.cuda.device(dev):
+    with _on(dev):
         check(lib().lift_partial_dot(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), int(bool(contract)), _stream(dev)))
     return out
 
@@ -239,7 +256,7 @@ def lift_dot_listing1(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None
         out = torch.empty((), dtype=torch.float32, device=dev)
     L = lib()
     n = x.numel()
-    with torch.cuda.device(dev):
+    with _on(dev):
         ws = _workspace("listing1", dev, L.lift_dot_listing1_workspace_bytes(n), zero=False)
         check(L.lift_dot_listing1(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
                                   int(bool(contract)), _stream(dev)))
@@ -273,7 +290,7 @@ def lift_sgemv(alpha: float, A: torch.Tensor, x: torch.Tensor, beta: float = 0.0
         raise ValueError("x / y length does not match op(A)")
     L = lib()
     need = L.lift_sgemv_workspace_bytes(lay, int(bool(trans)), m, n)
-    with torch.cuda.device(dev):
+    with _on(dev):
         ws = _workspace("sgemv", dev, need, zero=True) if need else None
         check(L.lift_sgemv(lay, int(bool(trans)), m, n, float(alpha), A.data_ptr(), ld, x.data_ptr(), float(beta),
                            y.data_ptr(), ws.data_ptr() if ws is not None else None, ws.numel() if ws is not None else 0,

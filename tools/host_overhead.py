@@ -29,6 +29,8 @@ calls = {
     "lift_atax C ABI": lambda: L.lift_atax(64, 1024, A.data_ptr(), x.data_ptr(), yt.data_ptr(), ws_atax.data_ptr(),
                                            ws_atax.numel(), s),
     "lift.lift_gemv (binding)": lambda: lift.lift_gemv(A, x, out=y),
+    "lift.lift_dot (binding)": lambda: lift.lift_dot(x, x, out=r),
+    "lift.lift_atax (binding)": lambda: lift.lift_atax(A, x, out=yt),
 }
 for name, fn in calls.items():
     for _ in range(200):
