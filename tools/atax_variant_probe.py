@@ -25,6 +25,10 @@ VARIANTS = {
                CASES],
     # deeper ring (more bytes in flight per SM)
     "ring160": [("constexpr size_t kFusedRingTarget = 112 * 1024;", "constexpr size_t kFusedRingTarget = 160 * 1024;")],
+    # column pass (transposed SGEMV, two-pass ATAX): fewer row splits, more rows per block
+    "splits_div2": [("    int64_t S = (int64_t)d.sms * per_sm / cblocks;", "    int64_t S = (int64_t)d.sms * per_sm / cblocks / 2;")],
+    "splits_x2": [("    int64_t S = (int64_t)d.sms * per_sm / cblocks;", "    int64_t S = (int64_t)d.sms * per_sm / cblocks * 2;")],
+    "splits_div4": [("    int64_t S = (int64_t)d.sms * per_sm / cblocks;", "    int64_t S = (int64_t)d.sms * per_sm / cblocks / 4;")],
     # 16 KiB stages (more, smaller bulk copies; twice the steps)
     "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
 }
@@ -47,15 +51,19 @@ def patched(name):
     return d
 
 
+TIMER = "ab_atax.py"
+if "--colpass" in sys.argv:
+    sys.argv.remove("--colpass")
+    TIMER = "ab_colpass.py"
 names = sys.argv[1:] or list(VARIANTS)
 res = {}
 for name in names:
     d = patched(name)
     print(f"== {name}", flush=True)
     out = os.path.join(d, "out.npz")
-    subprocess.run([sys.executable, os.path.join(ROOT, "tools", "ab_atax.py"), out], cwd=d, check=True)
+    subprocess.run([sys.executable, os.path.join(ROOT, "tools", TIMER), out], cwd=d, check=True)
     res[name] = np.load(out)
 if "lib" in res:
     for name, r in res.items():
-        same = [k for k in r.files if k.startswith("y_") and np.array_equal(r[k], res["lib"][k])]
+        same = [k for k in r.files if not k.startswith("t_") and np.array_equal(r[k], res["lib"][k])]
         print(name, "bitwise equal to lib at:", ", ".join(s[2:] for s in same))
