@@ -345,13 +345,77 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
     return true;
 }
 
-bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
-    FusedPlan p;
-    return aligned16 && m > 0 && fused_plan(n, &p);
+// ---------------------------------------------------------------------------
+// Wide rows (n > 16384: two rows and x no longer fit one block's ring): the
+// columns are split over a thread-block cluster of C blocks.  Block r of a
+// cluster owns the column slice [r*n/C, (r+1)*n/C) of every row its cluster
+// streams, with x and y of that slice in registers; a row's dot is the
+// fixed-order sum of the C blocks' slice dots.
+// ---------------------------------------------------------------------------
+struct WidePlan {
+    int clu;      // cluster size C (2, 4, 8 or 16)
+    int qc;       // float4 columns per thread within the slice (1 or 2)
+    int nst;      // ring stages (kWideRows row slices each)
+    size_t hdr;   // mbarriers + pushed warp sums
+    size_t smem;  // dynamic smem bytes
+};
+
+constexpr int kWideRows = 4;  // rows per step: one cluster barrier per 4 rows
+constexpr int kWideBufs = 4;  // pushed-sum buffers (a producer is at most 3 steps ahead of a reader)
+
+static size_t wide_sums_bytes(int c) { return 8 * kWideBufs + (size_t)kWideBufs * kWideRows * c * kFusedWarps * 4; }
+
+static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) {
+    FusedPlan narrow;
+    if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it
+    if (tune.l2a > 0 || tune.clu > 1 || tune.clu < 0) return false;     // no L2 prefetch / cluster second stage
+    for (int c = 2; c <= kFusedMaxCluster; c *= 2) {
+        if (n % (4 * c) != 0) return false;  // every slice a whole number of float4 columns
+        const int64_t nvs = n / c / 4;
+        if (nvs > 2 * (int64_t)kFusedThreads) continue;
+        p->clu = c;
+        p->qc = nvs <= kFusedThreads ? 1 : 2;
+        const size_t stage = (size_t)kWideRows * (size_t)(n / c) * 4;
+        // as many stages as the shared-memory budget holds: a stage is refilled only
+        // once every row of it has been used, so the ring is what keeps HBM busy
+        const size_t hdr = (8 * kFusedMaxStages + wide_sums_bytes(c) + 127) / 128 * 128;
+        int64_t nst = (int64_t)(((size_t)kFusedSmemBudget - hdr) / stage);
+        if (nst < 2) nst = 2;
+        if (nst > kFusedMaxStages) nst = kFusedMaxStages;
+        if (tune.nst != 0) {
+            if (tune.nst < 2 || tune.nst > kFusedMaxStages) return false;
+            nst = tune.nst;
+        }
+        p->nst = (int)nst;
+        p->hdr = (8 * kFusedMaxStages + wide_sums_bytes(c) + 127) / 128 * 128;
+        const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
+        p->smem = p->hdr + (ring > tile ? ring : tile);
+        return p->smem <= (size_t)kFusedSmemBudget;
+    }
+    return false;
 }
 
+bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
+    FusedPlan p;
+    WidePlan w;
+    return aligned16 && m > 0 && (fused_plan(n, &p) || wide_plan(n, &w));
+}
+
+// algo = auto: the single-block kernel from n = 256 up; the cluster kernel only
+// where it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
+// clusters of at most 8 blocks whose threads all own 2 float4 columns, e.g.
+// 8192x32768 271 vs 309 us; narrower slices or 16-block clusters lose)
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
-    return atax_fused_supported(m, n, aligned16) && n >= kFusedMinN;
+    if (!atax_fused_supported(m, n, aligned16) || n < kFusedMinN) return false;
+    FusedPlan p;
+    if (fused_plan(n, &p)) return true;
+    WidePlan w;
+    return wide_plan(n, &w) && w.clu <= 8 && (n / w.clu / 4) % (2 * kFusedThreads) == 0;
+}
+
+bool atax_fused_exchange_supported(int64_t m, int64_t n, bool aligned16) {
+    FusedPlan p;
+    return aligned16 && m > 0 && fused_plan(n, &p) && n >= kFusedMinN;
 }
 
 // Fixed-order column sum of the vector columns [c0, c1) over S partial rows,
@@ -896,6 +960,230 @@ static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m,
                               rows_are_lines(P, n), clu);
 }
 
+// Wide-row fused ATAX (see WidePlan).  Cluster kc of K streams the row groups
+// (CR consecutive rows) kc, kc+K, ...; its block r reads the groups' column
+// slice r (CR bulk copies per stage into a ring, as k_atax_fused).
+// Step k: the slice dots of group k are reduced per warp and PUSHED into
+// every block's sum buffer k % 4 with asynchronous remote stores
+// (st.async ... mbarrier::complete_tx), each completing bytes on the
+// destination's "sums full" mbarrier of that buffer, which its owner arms with
+// the step's expected bytes.  Then the block waits for buffer (k-1) % 4 to be
+// full (every block's group k-1 sums landed) and applies group k-1's rank-1
+// updates: t_r = pairwise tree over row r's C x 16 sums in (block, warp)
+// order.  No cluster barrier in the loop: blocks drift freely, and a producer
+// can be at most three steps ahead of any reader, so four buffers suffice.
+// Second stage: partial y rows P[kc][slice] -> grid barrier -> fixed-order
+// column sum over the K cluster rows.
+template <int QC, int CR, int C>
+__global__ void __launch_bounds__(kFusedThreads, 1)
+    k_atax_fused_wide(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A,
+                      const float *__restrict__ x, float *__restrict__ P, float *__restrict__ y,
+                      unsigned int *__restrict__ gbar, bool discard_partials) {
+    extern __shared__ __align__(128) unsigned char smem[];
+    uint64_t *full = reinterpret_cast<uint64_t *>(smem);
+    uint64_t *sfull = full + kFusedMaxStages;                              // [4]
+    float *sums = reinterpret_cast<float *>(sfull + kWideBufs);            // [4][CR][C][16]
+    float *stage0 = reinterpret_cast<float *>(smem + hdr);
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int tid = threadIdx.x;
+    const int r = (int)cluster_ctarank();
+    const int64_t K = cluster_count_x(), kc = cluster_id_x();
+    const int64_t nc = n / C, nvs = nc / 4, col0 = (int64_t)r * nc;
+    const int64_t groups = (m + CR - 1) / CR;
+    const int64_t nstages = kc < groups ? (groups - kc + K - 1) / K : 0;
+    const size_t stage_floats = (size_t)CR * nc;
+    constexpr int SB = CR * C * kFusedWarps;  // floats per sum buffer
+    constexpr uint32_t kStepBytes = SB * 4;   // bytes every block pushes into one buffer per step
+    auto stage_rows = [&](int64_t j) -> int {
+        if (j >= nstages) return 0;
+        const int64_t r0 = (j * K + kc) * CR;
+        return (int)(m - r0 < CR ? m - r0 : CR);
+    };
+    auto issue_stage = [&](int64_t j, int slot) {
+        const int rows = stage_rows(j);
+        const int64_t r0 = (j * K + kc) * CR;
+        mbar_arrive_expect_tx(full + slot, (uint32_t)(rows * nc * 4));
+        for (int i = 0; i < rows; ++i)
+            bulk_g2s(stage0 + (size_t)slot * stage_floats + (size_t)i * nc, A + (r0 + i) * n + col0,
+                     (uint32_t)(nc * 4), full + slot);
+    };
+    if (tid == 0) {
+        for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
+        for (int i = 0; i < kWideBufs; ++i) mbar_init(sfull + i, 1);
+        fence_mbar_init();
+    }
+    // every block's barriers are initialised and it is running before anyone
+    // pushes into its shared memory
+    cluster_sync();
+    if (tid == 0)
+        for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
+
+    const float4 *x4 = reinterpret_cast<const float4 *>(x + col0);
+    float4 xr[QC], yr[QC];
+#pragma unroll
+    for (int q = 0; q < QC; ++q) {
+        const int64_t c = tid + (int64_t)kFusedThreads * q;
+        xr[q] = c < nvs ? ld_ro4(x4 + c) : zero4();
+        yr[q] = zero4();
+    }
+    int sb = 0, psb = 0, slot = 0, pslot = 0, prow = 0;
+    uint32_t phase = 0, sphase = 0, psphase = 0;  // ring parity; sum-buffer parity of steps k and k-1
+    int64_t k = 0;
+    float4 ra[CR][QC], rb2[CR][QC];
+    auto step = [&](float4(&cur)[CR][QC], float4(&prev)[CR][QC]) -> bool {
+        const int rows = stage_rows(k);
+        __syncthreads();  // this block: step k-1's ring slot and sum buffer k-1 consumed
+        if (tid == 0) {
+            if (prow > 0 && k - 1 + nst < nstages) issue_stage(k - 1 + nst, pslot);
+            if (rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);  // arm buffer k % 4
+        }
+        if (rows > 0) {
+            mbar_wait_parity(full + slot, phase);
+            const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)slot * stage_floats);
+            float d[CR];
+#pragma unroll
+            for (int i = 0; i < CR; ++i) {
+                float4 acc = zero4();
+#pragma unroll
+                for (int q = 0; q < QC; ++q) {
+                    const int64_t c = tid + (int64_t)kFusedThreads * q;
+                    cur[i][q] = (i < rows && c < nvs) ? S4[(int64_t)i * nvs + c] : zero4();
+                    fma4(acc, cur[i][q], xr[q]);
+                }
+                d[i] = hsum4(acc);
+            }
+            // row i's warp sum ends in lanes [i*32/CR, (i+1)*32/CR): lane i*32/CR + b
+            // pushes it to block b (and b + 32/CR, ... when C > 32/CR)
+            const float dr = row_butterfly<CR>(d, lane);
+            const int li = lane & (32 / CR - 1), row = lane / (32 / CR);
+            const uint32_t la = smem_u32(sums + sb * SB + (row * C + r) * kFusedWarps + warp);
+            const uint32_t lb = smem_u32(sfull + sb);
+#pragma unroll
+            for (int b = 0; b < C; b += 32 / CR)
+                if (b + li < C)
+                    st_async_dsmem1(dsmem_addr_raw(la, (uint32_t)(b + li)), dr, dsmem_addr_raw(lb, (uint32_t)(b + li)));
+        }
+        if (prow > 0) {
+            mbar_wait_parity(sfull + psb, psphase);  // every block's group k-1 sums are here
+            // t_r = pairwise tree over row r's C x 16 sums in (block, warp) order (=
+            // a pairwise tree over the blocks of each block's pairwise tree over its
+            // warps).  The CR rows are folded over the warp: 32/CR lanes per row, each
+            // lane's 2C contiguous sums are the lowest tree levels, a butterfly over
+            // the row's lanes the rest; then every lane takes the CR results.
+            constexpr int LPR = 32 / CR, VPL = C * kFusedWarps / LPR;
+            const int row = lane / LPR, li = lane % LPR;
+            const float4 *pb4 = reinterpret_cast<const float4 *>(sums + psb * SB + row * C * kFusedWarps + li * VPL);
+            float v[VPL];
+#pragma unroll
+            for (int u = 0; u < VPL / 4; ++u) {
+                const float4 f = pb4[u];
+                v[4 * u] = f.x;
+                v[4 * u + 1] = f.y;
+                v[4 * u + 2] = f.z;
+                v[4 * u + 3] = f.w;
+            }
+            float tv = pair_tree<VPL>(v);
+#pragma unroll
+            for (int o = 1; o < LPR; o <<= 1) tv = __fadd_rn(tv, __shfl_xor_sync(0xffffffffu, tv, o));
+#pragma unroll
+            for (int i = 0; i < CR; ++i) {
+                const float t = __shfl_sync(0xffffffffu, tv, i * LPR);
+                if (i < prow)
+#pragma unroll
+                    for (int q = 0; q < QC; ++q) fma4s(yr[q], prev[i][q], t);
+            }
+        }
+        if (rows == 0) return true;
+        prow = rows;
+        pslot = slot;
+        if (++slot == nst) {
+            slot = 0;
+            phase ^= 1u;
+        }
+        psb = sb;
+        psphase = sphase;
+        if (++sb == kWideBufs) {
+            sb = 0;
+            sphase ^= 1u;
+        }
+        ++k;
+        return false;
+    };
+    for (;;) {
+        if (step(ra, rb2)) break;
+        if (step(rb2, ra)) break;
+    }
+    cluster_sync();  // no block leaves while a peer's pushes or reads may still involve it
+    // partial y row of this cluster, this block's slice
+    float4 *P4 = reinterpret_cast<float4 *>(P + kc * n + col0);
+#pragma unroll
+    for (int q = 0; q < QC; ++q) {
+        const int64_t c = tid + (int64_t)kFusedThreads * q;
+        if (c < nvs) P4[c] = yr[q];
+    }
+    grid_barrier(gbar);
+    const int64_t nv = n / 4;
+    const bool lines = discard_partials;
+    const int64_t unit = lines ? 8 : 1, nu = (nv + unit - 1) / unit;
+    int64_t c0 = unit * (nu * blockIdx.x / gridDim.x), c1 = unit * (nu * (blockIdx.x + 1) / gridDim.x);
+    if (c1 > nv) c1 = nv;
+    colsum_slice<8>((int)K, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0), lines);
+    grid_depart(gbar);
+}
+
+template <int QC, int CR, int C>
+static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, int64_t n, const float *A,
+                            const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s) {
+    auto k = k_atax_fused_wide<QC, CR, C>;
+    cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
+    if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+    if (e != cudaSuccess) return e;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeClusterDimension;
+    attr[0].val.clusterDim.x = (unsigned)C;
+    attr[0].val.clusterDim.y = 1;
+    attr[0].val.clusterDim.z = 1;
+    cudaLaunchConfig_t cfg = {};
+    cfg.blockDim = dim3(kFusedThreads);
+    cfg.dynamicSmemBytes = p.smem;
+    cfg.stream = s;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    cfg.gridDim = dim3((unsigned)(C * (d.sms / C)));
+    // every cluster resident at once (the grid barrier needs it): as many clusters
+    // as the occupancy calculator says fit, cached per (device, shape)
+    struct Entry {
+        int dev, clu, qc, nst;
+        size_t smem;
+        int nc;
+    };
+    static Entry cache[16];
+    static int used = 0;
+    static std::mutex mu;
+    int nc = -1;
+    {
+        std::lock_guard<std::mutex> lock(mu);
+        for (int i = 0; i < used; ++i)
+            if (cache[i].dev == d.device && cache[i].clu == C && cache[i].qc == QC && cache[i].nst == p.nst &&
+                cache[i].smem == p.smem)
+                nc = cache[i].nc;
+        if (nc < 0) {
+            if (cudaOccupancyMaxActiveClusters(&nc, k, &cfg) != cudaSuccess) {
+                (void)cudaGetLastError();
+                nc = 0;
+            }
+            if (used < 16) cache[used++] = Entry{d.device, C, QC, p.nst, p.smem, nc};
+        }
+    }
+    int64_t K = nc;
+    if (K < 1) return cudaErrorInvalidConfiguration;
+    if (K > kMaxSplits) K = kMaxSplits;
+    const int64_t groups = (m + kWideRows - 1) / kWideRows;
+    if (K > groups) K = groups;
+    cfg.gridDim = dim3((unsigned)(K * C));
+    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
+}
+
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     cudaFuncAttributes a;
     cudaError_t e = cudaFuncGetAttributes(&a, k_atax_fused<1, 4>);
@@ -905,6 +1193,11 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
+#define LIFT_WIDE_PRELOAD(QC, C) \
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<QC, kWideRows, C>);
+    LIFT_WIDE_PRELOAD(1, 2) LIFT_WIDE_PRELOAD(2, 2) LIFT_WIDE_PRELOAD(1, 4) LIFT_WIDE_PRELOAD(2, 4)
+    LIFT_WIDE_PRELOAD(1, 8) LIFT_WIDE_PRELOAD(2, 8) LIFT_WIDE_PRELOAD(1, 16) LIFT_WIDE_PRELOAD(2, 16)
+#undef LIFT_WIDE_PRELOAD
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<4, 256, 8>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<1, 256, 8>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_colsum<4>);
@@ -916,7 +1209,20 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
                               void *ws, cudaStream_t s, Exch ex, int dst, int blocks, FusedTuning tune) {
     if (n == 0) return cudaSuccess;
     FusedPlan p;
-    if (!fused_plan(n, &p, tune)) return cudaErrorInvalidValue;
+    if (!fused_plan(n, &p, tune)) {
+        // wide rows: the cluster kernel (single rank, grid from the cluster occupancy)
+        WidePlan w;
+        if (ex.world != 0 || blocks > 0 || !wide_plan(n, &w, tune)) return cudaErrorInvalidValue;
+        if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
+        unsigned int *gbar = static_cast<unsigned int *>(ws);
+        float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
+#define LIFT_WIDE_CASE(QC, C) \
+    if (w.qc == QC && w.clu == C) return run_wide<QC, kWideRows, C>(d, w, m, n, A, x, P, y, gbar, s);
+        LIFT_WIDE_CASE(1, 2) LIFT_WIDE_CASE(2, 2) LIFT_WIDE_CASE(1, 4) LIFT_WIDE_CASE(2, 4)
+        LIFT_WIDE_CASE(1, 8) LIFT_WIDE_CASE(2, 8) LIFT_WIDE_CASE(1, 16) LIFT_WIDE_CASE(2, 16)
+#undef LIFT_WIDE_CASE
+        return cudaErrorInvalidValue;
+    }
     if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
     unsigned int *gbar = static_cast<unsigned int *>(ws);
     float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);

@@ -487,7 +487,7 @@ int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float
     if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
     const bool aligned = ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
                            reinterpret_cast<uintptr_t>(y)) & 15) == 0;
-    if (n > 0 && !lift::atax_fused_preferred(m > 0 ? m : 1, n, aligned)) return LIFT_ERR_BAD_SIZE;
+    if (n > 0 && !lift::atax_fused_exchange_supported(m > 0 ? m : 1, n, aligned)) return LIFT_ERR_BAD_SIZE;
     if (n > 0 && (y == nullptr || x == nullptr || (m > 0 && A == nullptr))) return LIFT_ERR_NULL_PTR;
     if (workspace == nullptr || workspace_bytes < lift_atax_workspace_bytes(m, n) ||
         (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)

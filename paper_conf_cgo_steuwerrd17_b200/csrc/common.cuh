@@ -228,6 +228,16 @@ __device__ __forceinline__ uint32_t dsmem_addr_raw(uint32_t local_smem, uint32_t
     asm volatile("mapa.shared::cluster.u32 %0, %1, %2;" : "=r"(a) : "r"(local_smem), "r"(rank));
     return a;
 }
+// Asynchronous remote store that completes `4` transaction bytes on the
+// destination CTA's mbarrier when the value lands (no membar needed).
+__device__ __forceinline__ void st_async_dsmem1(uint32_t addr, float v, uint32_t remote_bar) {
+    asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.b32 [%0], %1, [%2];" ::"r"(addr),
+                 "r"(__float_as_uint(v)), "r"(remote_bar)
+                 : "memory");
+}
+__device__ __forceinline__ void st_dsmem1(uint32_t addr, float v) {
+    asm volatile("st.shared::cluster.f32 [%0], %1;" ::"r"(addr), "f"(v) : "memory");
+}
 __device__ __forceinline__ float4 ld_dsmem4(uint32_t addr) {
     float4 v;
     asm volatile("ld.shared::cluster.v4.f32 {%0, %1, %2, %3}, [%4];"

@@ -330,13 +330,31 @@ def test_gesummv_reductions_bitwise(cuda_device):
 ATAX_SHAPES = [(1, 1), (5, 3), (3, 7), (64, 32), (1000, 300), (300, 1001), (4096, 4096), (2000, 16384), (100, 20000)]
 
 
+def fused_supported(n: int) -> bool:
+    """Shapes the single-pass ATAX accepts (16-B aligned operands): n % 4 == 0 and
+    either n <= 16384 (one block per row) or a cluster of C = 2..16 blocks whose
+    column slices are whole float4 columns, at most 1024 float4 each."""
+    if n % 4:
+        return False
+    if n <= 16384:
+        return True
+    c = 2
+    while c <= 16:
+        if n % (4 * c):
+            return False
+        if n // c // 4 <= 1024:
+            return True
+        c *= 2
+    return False
+
+
 @pytest.mark.parametrize("m,n", ATAX_SHAPES)
 @pytest.mark.parametrize("algo", ["auto", "fused", "twopass"])
 def test_atax_parity(cuda_device, m, n, algo):
     A = rand(synth.SEED_A, (m, n))
     x = rand(synth.SEED_X, (n,))
     Ad, xd = dev_np(A, cuda_device), dev_np(x, cuda_device)
-    if algo == "fused" and n % 4 != 0 or (algo == "fused" and n > 16384):
+    if algo == "fused" and not fused_supported(n):
         with pytest.raises(lift.LiftError):
             lift.lift_atax(Ad, xd, algo=algo)
         return
@@ -373,6 +391,45 @@ def test_atax_fused_tuning(cuda_device):
         for bad in (dict(nst=1), dict(nst=17), dict(l2_ahead=65), dict(cyclic=2)):
             with pytest.raises(lift.LiftError):
                 lift.lift_atax_fused_tuned(A, x, **bad)
+
+
+WIDE_SHAPES = [(1, 16416), (3, 20000), (300, 32768), (1001, 24576), (64, 65536), (777, 16416), (2048, 32768)]
+
+
+@pytest.mark.parametrize("m,n", WIDE_SHAPES)
+def test_atax_fused_wide(cuda_device, m, n):
+    """Single-pass ATAX for rows wider than one block can ring-buffer
+    (n > 16384): the columns split over a thread-block cluster, row dots
+    pushed as warp sums into every block's shared memory by asynchronous
+    remote stores.  Oracle tolerance, bitwise repeatable, chosen by
+    algo="auto" where it is the faster algorithm (n = 32768 here), and within
+    tolerance of the two-pass algorithm."""
+    assert fused_supported(n)
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+    got = lift.lift_atax(A, x, algo="fused")
+    assert_tol(got.cpu().numpy(), ref, mag, f"atax wide {m}x{n}")
+    for _ in range(2):
+        assert torch.equal(lift.lift_atax(A, x, algo="fused"), got)
+    auto = lift.lift_atax(A, x)  # the single pass where it beats the two-pass algorithm
+    assert_tol(auto.cpu().numpy(), ref, mag, f"atax auto {m}x{n}")
+    if n in (32768,):
+        assert torch.equal(auto, got)
+    assert_tol(lift.lift_atax(A, x, algo="twopass").cpu().numpy(), ref, mag, f"atax twopass {m}x{n}")
+
+
+def test_atax_fused_wide_rejects(cuda_device):
+    """Wide rows whose cluster slices would not be whole float4 columns stay on
+    the two-pass algorithm (auto) and are refused by algo="fused"."""
+    for n in (16392, 16388, 20004, 16400):
+        assert not fused_supported(n)
+        A = synth.torch_matrix_rows(synth.SEED_A, n, 0, 5, device=cuda_device)
+        x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+        with pytest.raises(lift.LiftError):
+            lift.lift_atax(A, x, algo="fused")
+        ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+        assert_tol(lift.lift_atax(A, x).cpu().numpy(), ref, mag, f"atax auto {n}")
 
 
 @pytest.mark.parametrize("cluster", [1, 2, 4, 8, 16])
