@@ -363,7 +363,9 @@ struct WidePlan {
 constexpr int kWideRows = 4;  // rows per step: one cluster barrier per 4 rows
 constexpr int kWideBufs = 4;  // pushed-sum buffers (a producer is at most 3 steps ahead of a reader)
 
-static size_t wide_sums_bytes(int c) { return 8 * kWideBufs + (size_t)kWideBufs * kWideRows * c * kFusedWarps * 4; }
+static size_t wide_sums_bytes(int c) {
+    return 8 * kWideBufs + 4 * kFusedMaxStages + (size_t)kWideBufs * kWideRows * c * kFusedWarps * 4;
+}
 
 static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) {
     FusedPlan narrow;
@@ -404,7 +406,7 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
 // algo = auto: the single-block kernel from n = 256 up; the cluster kernel only
 // where it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
 // clusters of at most 8 blocks whose threads all own 2 float4 columns, e.g.
-// 8192x32768 271 vs 309 us; narrower slices or 16-block clusters lose)
+// 8192x32768 259 vs 309 us; narrower slices or 16-block clusters lose)
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     if (!atax_fused_supported(m, n, aligned16) || n < kFusedMinN) return false;
     FusedPlan p;
@@ -972,6 +974,7 @@ static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m,
 // updates: t_r = pairwise tree over row r's C x 16 sums in (block, warp)
 // order.  No cluster barrier in the loop: blocks drift freely, and a producer
 // can be at most three steps ahead of any reader, so four buffers suffice.
+// No block barrier either: the last warp done with a ring slot refills it.
 // Second stage: partial y rows P[kc][slice] -> grid barrier -> fixed-order
 // column sum over the K cluster rows.
 template <int QC, int CR, int C>
@@ -982,7 +985,8 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     uint64_t *sfull = full + kFusedMaxStages;                              // [4]
-    float *sums = reinterpret_cast<float *>(sfull + kWideBufs);            // [4][CR][C][16]
+    unsigned int *used = reinterpret_cast<unsigned int *>(sfull + kWideBufs);  // [16] warps done with a slot
+    float *sums = reinterpret_cast<float *>(used + kFusedMaxStages);       // [4][CR][C][16]
     float *stage0 = reinterpret_cast<float *>(smem + hdr);
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int tid = threadIdx.x;
@@ -1010,6 +1014,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     if (tid == 0) {
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         for (int i = 0; i < kWideBufs; ++i) mbar_init(sfull + i, 1);
+        for (int i = 0; i < kFusedMaxStages; ++i) used[i] = 0u;
         fence_mbar_init();
     }
     // every block's barriers are initialised and it is running before anyone
@@ -1032,11 +1037,10 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     float4 ra[CR][QC], rb2[CR][QC];
     auto step = [&](float4(&cur)[CR][QC], float4(&prev)[CR][QC]) -> bool {
         const int rows = stage_rows(k);
-        __syncthreads();  // this block: step k-1's ring slot and sum buffer k-1 consumed
-        if (tid == 0) {
-            if (prow > 0 && k - 1 + nst < nstages) issue_stage(k - 1 + nst, pslot);
-            if (rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);  // arm buffer k % 4
-        }
+        // no block barrier in the loop: warps of a block are at most one step apart
+        // (a warp at step k has seen every warp's group k-1 push), so warp 0 may arm
+        // buffer k % 4 (last used by step k-4, waited for by every warp by step k-3)
+        if (tid == 0 && rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);
         if (rows > 0) {
             mbar_wait_parity(full + slot, phase);
             const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)slot * stage_floats);
@@ -1051,6 +1055,15 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
                     fma4(acc, cur[i][q], xr[q]);
                 }
                 d[i] = hsum4(acc);
+            }
+            // this warp is done with the ring slot: the last of the 16 warps to get here
+            // refills it with stage k + nst (acq_rel orders every warp's reads before it)
+            __syncwarp();
+            if (lane == 0) {
+                if (atom_acq_rel_add_cta_shared(used + slot, 1u) == kFusedWarps - 1) {
+                    used[slot] = 0u;
+                    if (k + nst < nstages) issue_stage(k + nst, slot);
+                }
             }
             // row i's warp sum ends in lanes [i*32/CR, (i+1)*32/CR): lane i*32/CR + b
             // pushes it to block b (and b + 32/CR, ... when C > 32/CR)

@@ -122,6 +122,13 @@ __device__ __forceinline__ uint32_t smem_u32(const void *p) {
     return static_cast<uint32_t>(__cvta_generic_to_shared(p));
 }
 
+// CTA-scope acquire-release add on a shared-memory counter ("last arriver" hand-offs)
+__device__ __forceinline__ unsigned int atom_acq_rel_add_cta_shared(unsigned int *p, unsigned int v) {
+    unsigned int r;
+    asm volatile("atom.acq_rel.cta.shared::cta.add.u32 %0, [%1], %2;" : "=r"(r) : "r"(smem_u32(p)), "r"(v) : "memory");
+    return r;
+}
+
 __device__ __forceinline__ void mbar_init(uint64_t *bar, uint32_t count) {
     asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
 }
