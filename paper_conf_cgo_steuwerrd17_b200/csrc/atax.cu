@@ -354,13 +354,14 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
 // ---------------------------------------------------------------------------
 struct WidePlan {
     int clu;      // cluster size C (2, 4, 8 or 16)
-    int qc;       // float4 columns per thread within the slice (1 or 2)
-    int nst;      // ring stages (kWideRows row slices each)
+    int qc;       // float4 columns per thread within the slice (1, 2 or 4)
+    int cr;       // rows per step (4, or 2 when qc = 4: registers)
+    int nst;      // ring stages (cr row slices each)
     size_t hdr;   // mbarriers + pushed warp sums
     size_t smem;  // dynamic smem bytes
 };
 
-constexpr int kWideRows = 4;  // rows per step: one cluster barrier per 4 rows
+constexpr int kWideRows = 4;  // rows per step (at most)
 constexpr int kWideBufs = 4;  // pushed-sum buffers (a producer is at most 3 steps ahead of a reader)
 
 static size_t wide_sums_bytes(int c) {
@@ -371,13 +372,19 @@ static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) 
     FusedPlan narrow;
     if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it
     if (tune.l2a > 0 || tune.clu > 1 || tune.clu < 0) return false;     // no L2 prefetch / cluster second stage
-    for (int c = 2; c <= kFusedMaxCluster; c *= 2) {
-        if (n % (4 * c) != 0) return false;  // every slice a whole number of float4 columns
+    // clusters of 8 measured fastest (profiles/r01z_atax_wide_cluster_probe.txt: 4 and
+    // 16 lose even with more SMs or narrower slices); other sizes only where 8 cannot
+    // split the row into whole float4 slices of at most 2048 float4
+    int order[4] = {8, 2, 4, 16};
+    for (int c : order) {
+        if (n % (4 * c) != 0) continue;  // every slice a whole number of float4 columns
         const int64_t nvs = n / c / 4;
-        if (nvs > 2 * (int64_t)kFusedThreads) continue;
+        if (nvs > 4 * (int64_t)kFusedThreads) continue;
+        if (c == 2 && n % 16 == 0 && n / 16 <= 4 * (int64_t)kFusedThreads) continue;  // prefer 4 over 2
         p->clu = c;
-        p->qc = nvs <= kFusedThreads ? 1 : 2;
-        const size_t stage = (size_t)kWideRows * (size_t)(n / c) * 4;
+        p->qc = nvs <= kFusedThreads ? 1 : (nvs <= 2 * kFusedThreads ? 2 : 4);
+        p->cr = p->qc == 4 ? 2 : kWideRows;
+        const size_t stage = (size_t)p->cr * (size_t)(n / c) * 4;
         // as many stages as the shared-memory budget holds: a stage is refilled only
         // once every row of it has been used, so the ring is what keeps HBM busy
         const size_t hdr = (8 * kFusedMaxStages + wide_sums_bytes(c) + 127) / 128 * 128;
@@ -389,7 +396,7 @@ static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) 
             nst = tune.nst;
         }
         p->nst = (int)nst;
-        p->hdr = (8 * kFusedMaxStages + wide_sums_bytes(c) + 127) / 128 * 128;
+        p->hdr = hdr;
         const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
         p->smem = p->hdr + (ring > tile ? ring : tile);
         return p->smem <= (size_t)kFusedSmemBudget;
@@ -405,14 +412,14 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
 
 // algo = auto: the single-block kernel from n = 256 up; the cluster kernel only
 // where it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
-// clusters of at most 8 blocks whose threads all own 2 float4 columns, e.g.
-// 8192x32768 259 vs 309 us; narrower slices or 16-block clusters lose)
+// clusters of 8 blocks whose slices are whole multiples of 512 float4, e.g.
+// 8192x32768 259 vs 309 us, 4096x65536 245 vs 323; other shapes lose)
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     if (!atax_fused_supported(m, n, aligned16) || n < kFusedMinN) return false;
     FusedPlan p;
     if (fused_plan(n, &p)) return true;
     WidePlan w;
-    return wide_plan(n, &w) && w.clu <= 8 && (n / w.clu / 4) % (2 * kFusedThreads) == 0;
+    return wide_plan(n, &w) && w.clu == 8 && (n / w.clu / 4) % kFusedThreads == 0;
 }
 
 bool atax_fused_exchange_supported(int64_t m, int64_t n, bool aligned16) {
@@ -1191,7 +1198,7 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
     int64_t K = nc;
     if (K < 1) return cudaErrorInvalidConfiguration;
     if (K > kMaxSplits) K = kMaxSplits;
-    const int64_t groups = (m + kWideRows - 1) / kWideRows;
+    const int64_t groups = (m + CR - 1) / CR;
     if (K > groups) K = groups;
     cfg.gridDim = dim3((unsigned)(K * C));
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
@@ -1206,10 +1213,12 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
-#define LIFT_WIDE_PRELOAD(QC, C) \
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<QC, kWideRows, C>);
-    LIFT_WIDE_PRELOAD(1, 2) LIFT_WIDE_PRELOAD(2, 2) LIFT_WIDE_PRELOAD(1, 4) LIFT_WIDE_PRELOAD(2, 4)
-    LIFT_WIDE_PRELOAD(1, 8) LIFT_WIDE_PRELOAD(2, 8) LIFT_WIDE_PRELOAD(1, 16) LIFT_WIDE_PRELOAD(2, 16)
+#define LIFT_WIDE_PRELOAD(QC, CR, C) \
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<QC, CR, C>);
+    LIFT_WIDE_PRELOAD(1, 4, 2) LIFT_WIDE_PRELOAD(2, 4, 2) LIFT_WIDE_PRELOAD(4, 2, 2)
+    LIFT_WIDE_PRELOAD(1, 4, 4) LIFT_WIDE_PRELOAD(2, 4, 4) LIFT_WIDE_PRELOAD(4, 2, 4)
+    LIFT_WIDE_PRELOAD(1, 4, 8) LIFT_WIDE_PRELOAD(2, 4, 8) LIFT_WIDE_PRELOAD(4, 2, 8)
+    LIFT_WIDE_PRELOAD(1, 4, 16) LIFT_WIDE_PRELOAD(2, 4, 16) LIFT_WIDE_PRELOAD(4, 2, 16)
 #undef LIFT_WIDE_PRELOAD
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<4, 256, 8>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<1, 256, 8>);
@@ -1229,10 +1238,12 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
         if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
         unsigned int *gbar = static_cast<unsigned int *>(ws);
         float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
-#define LIFT_WIDE_CASE(QC, C) \
-    if (w.qc == QC && w.clu == C) return run_wide<QC, kWideRows, C>(d, w, m, n, A, x, P, y, gbar, s);
-        LIFT_WIDE_CASE(1, 2) LIFT_WIDE_CASE(2, 2) LIFT_WIDE_CASE(1, 4) LIFT_WIDE_CASE(2, 4)
-        LIFT_WIDE_CASE(1, 8) LIFT_WIDE_CASE(2, 8) LIFT_WIDE_CASE(1, 16) LIFT_WIDE_CASE(2, 16)
+#define LIFT_WIDE_CASE(QC, CR, C) \
+    if (w.qc == QC && w.cr == CR && w.clu == C) return run_wide<QC, CR, C>(d, w, m, n, A, x, P, y, gbar, s);
+        LIFT_WIDE_CASE(1, 4, 2) LIFT_WIDE_CASE(2, 4, 2) LIFT_WIDE_CASE(4, 2, 2)
+        LIFT_WIDE_CASE(1, 4, 4) LIFT_WIDE_CASE(2, 4, 4) LIFT_WIDE_CASE(4, 2, 4)
+        LIFT_WIDE_CASE(1, 4, 8) LIFT_WIDE_CASE(2, 4, 8) LIFT_WIDE_CASE(4, 2, 8)
+        LIFT_WIDE_CASE(1, 4, 16) LIFT_WIDE_CASE(2, 4, 16) LIFT_WIDE_CASE(4, 2, 16)
 #undef LIFT_WIDE_CASE
         return cudaErrorInvalidValue;
     }

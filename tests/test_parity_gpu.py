@@ -332,20 +332,13 @@ ATAX_SHAPES = [(1, 1), (5, 3), (3, 7), (64, 32), (1000, 300), (300, 1001), (4096
 
 def fused_supported(n: int) -> bool:
     """Shapes the single-pass ATAX accepts (16-B aligned operands): n % 4 == 0 and
-    either n <= 16384 (one block per row) or a cluster of C = 2..16 blocks whose
-    column slices are whole float4 columns, at most 1024 float4 each."""
+    either n <= 16384 (one block per row) or a cluster of C in {2, 4, 8, 16}
+    blocks whose column slices are whole float4 columns, at most 2048 float4."""
     if n % 4:
         return False
     if n <= 16384:
         return True
-    c = 2
-    while c <= 16:
-        if n % (4 * c):
-            return False
-        if n // c // 4 <= 1024:
-            return True
-        c *= 2
-    return False
+    return any(n % (4 * c) == 0 and n // c // 4 <= 2048 for c in (2, 4, 8, 16))
 
 
 @pytest.mark.parametrize("m,n", ATAX_SHAPES)
@@ -393,7 +386,8 @@ def test_atax_fused_tuning(cuda_device):
                 lift.lift_atax_fused_tuned(A, x, **bad)
 
 
-WIDE_SHAPES = [(1, 16416), (3, 20000), (300, 32768), (1001, 24576), (64, 65536), (777, 16416), (2048, 32768)]
+WIDE_SHAPES = [(1, 16416), (3, 20000), (300, 32768), (1001, 24576), (64, 65536), (777, 16416), (2048, 32768),
+               (9, 16400), (5, 131072), (130, 49152)]
 
 
 @pytest.mark.parametrize("m,n", WIDE_SHAPES)
@@ -414,7 +408,7 @@ def test_atax_fused_wide(cuda_device, m, n):
         assert torch.equal(lift.lift_atax(A, x, algo="fused"), got)
     auto = lift.lift_atax(A, x)  # the single pass where it beats the two-pass algorithm
     assert_tol(auto.cpu().numpy(), ref, mag, f"atax auto {m}x{n}")
-    if n in (32768,):
+    if n in (32768, 65536, 49152):
         assert torch.equal(auto, got)
     assert_tol(lift.lift_atax(A, x, algo="twopass").cpu().numpy(), ref, mag, f"atax twopass {m}x{n}")
 
@@ -422,7 +416,7 @@ def test_atax_fused_wide(cuda_device, m, n):
 def test_atax_fused_wide_rejects(cuda_device):
     """Wide rows whose cluster slices would not be whole float4 columns stay on
     the two-pass algorithm (auto) and are refused by algo="fused"."""
-    for n in (16392, 16388, 20004, 16400):
+    for n in (16392, 16388, 20004):
         assert not fused_supported(n)
         A = synth.torch_matrix_rows(synth.SEED_A, n, 0, 5, device=cuda_device)
         x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
