@@ -29,6 +29,12 @@ VARIANTS = {
     "splits_div2": [("    int64_t S = (int64_t)d.sms * per_sm / cblocks;", "    int64_t S = (int64_t)d.sms * per_sm / cblocks / 2;")],
     "splits_x2": [("    int64_t S = (int64_t)d.sms * per_sm / cblocks;", "    int64_t S = (int64_t)d.sms * per_sm / cblocks * 2;")],
     "splits_div4": [("    int64_t S = (int64_t)d.sms * per_sm / cblocks;", "    int64_t S = (int64_t)d.sms * per_sm / cblocks / 4;")],
+    # wide-row cluster kernel with NO cross-block exchange (no arm, push or wait; WRONG results):
+    # the data path alone (ring, bulk copies, dots, updates) on the cluster launch
+    "wide_alone": [("            mbar_wait_parity(sfull + psb, psphase);  // every block's group k-1 sums are here", ""),
+                   ("                    st_async_dsmem1(dsmem_addr_raw(la, (uint32_t)(b + li)), dr, dsmem_addr_raw(lb, (uint32_t)(b + li)));",
+                    "                    if (dr == 1234.5f) sums[0] = dr;"),
+                   ("        if (tid == 0 && rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);", "")],
     # 16 KiB stages (more, smaller bulk copies; twice the steps)
     "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
 }
@@ -55,6 +61,9 @@ TIMER = "ab_atax.py"
 if "--colpass" in sys.argv:
     sys.argv.remove("--colpass")
     TIMER = "ab_colpass.py"
+if "--wide" in sys.argv:  # timing only (tools/atax_wide_probe.py), no bitwise comparison
+    sys.argv.remove("--wide")
+    TIMER = "atax_wide_probe.py"
 names = sys.argv[1:] or list(VARIANTS)
 res = {}
 for name in names:
@@ -62,7 +71,8 @@ for name in names:
     print(f"== {name}", flush=True)
     out = os.path.join(d, "out.npz")
     subprocess.run([sys.executable, os.path.join(ROOT, "tools", TIMER), out], cwd=d, check=True)
-    res[name] = np.load(out)
+    if TIMER != "atax_wide_probe.py":
+        res[name] = np.load(out)
 if "lib" in res:
     for name, r in res.items():
         same = [k for k in r.files if not k.startswith("t_") and np.array_equal(r[k], res["lib"][k])]

@@ -6,8 +6,8 @@ import sys
 
 import torch
 
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 sys.path.insert(0, os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, os.getcwd())  # run from a package root (this tree or a patched copy)
 import synth  # noqa: E402
 import paper_conf_cgo_steuwerrd17_b200 as lift  # noqa: E402
 from sweep import graph_time  # noqa: E402
@@ -15,7 +15,11 @@ from sweep import graph_time  # noqa: E402
 dev = torch.device("cuda:0")
 L2 = torch.cuda.get_device_properties(dev).L2_cache_size
 print(f"# {torch.cuda.get_device_name(dev)}  L2 {L2 >> 20} MiB", flush=True)
-for m, n in ((2048, 32768), (8192, 32768), (4096, 65536), (8192, 49152), (8192, 24576), (16384, 16416), (8192, 20000), (1024, 131072)):
+SHAPES = ((2048, 32768), (8192, 32768), (4096, 65536), (8192, 49152), (8192, 24576), (16384, 16416), (8192, 20000),
+          (1024, 131072))
+if os.environ.get("WIDE_QUICK"):
+    SHAPES = ((8192, 32768), (4096, 65536))
+for m, n in SHAPES:
     sets = max(2, -(-2 * L2 // (4 * m * n)))
     As = [synth.torch_matrix_rows(2 + 10 * k, n, 0, m, device=dev) for k in range(sets)]
     x = synth.torch_uniform(0, 0, n, device=dev)
