@@ -355,7 +355,8 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
 struct WidePlan {
     int clu;      // cluster size C (2, 4, 8 or 16)
     int qc;       // float4 columns per thread within the slice (1, 2 or 4)
-    int cr;       // rows per step (4, or 2 when qc = 4: registers)
+    int cr;       // rows per step (4; 1 in the lagged form)
+    bool lag;     // lagged form (qc = 4)
     int nst;      // ring stages (cr row slices each)
     size_t hdr;   // mbarriers + pushed warp sums
     size_t smem;  // dynamic smem bytes
@@ -363,9 +364,18 @@ struct WidePlan {
 
 constexpr int kWideRows = 4;  // rows per step (at most)
 constexpr int kWideBufs = 4;  // pushed-sum buffers (a producer is at most 3 steps ahead of a reader)
+// Lagged form (slices of more than 1024 float4, i.e. 32 KiB row slices): one
+// row per step, the rank-1 update of a row applied kWideLag steps after its
+// dot (its slice stays in the ring until then), so a block waits for the
+// peers' sums of row k-L, not k-1; 2L+2 sum buffers.  Narrower slices keep 4
+// rows per step in registers: one-row steps would stream 16 KiB copies.
+constexpr int kWideLag = 2;
+constexpr int kWideLagBufs = 2 * kWideLag + 2;
 
 static size_t wide_sums_bytes(int c) {
-    return 8 * kWideBufs + 4 * kFusedMaxStages + (size_t)kWideBufs * kWideRows * c * kFusedWarps * 4;
+    const size_t a = 8 * kWideBufs + 4 * kFusedMaxStages + (size_t)kWideBufs * kWideRows * c * kFusedWarps * 4;
+    const size_t b = 8 * kWideLagBufs + 4 * kFusedMaxStages + (size_t)kWideLagBufs * c * kFusedWarps * 4;
+    return a > b ? a : b;
 }
 
 static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) {
@@ -383,13 +393,15 @@ static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) 
         if (c == 2 && n % 16 == 0 && n / 16 <= 4 * (int64_t)kFusedThreads) continue;  // prefer 4 over 2
         p->clu = c;
         p->qc = nvs <= kFusedThreads ? 1 : (nvs <= 2 * kFusedThreads ? 2 : 4);
-        p->cr = p->qc == 4 ? 2 : kWideRows;
+        p->lag = p->qc == 4;
+        p->cr = p->lag ? 1 : kWideRows;
         const size_t stage = (size_t)p->cr * (size_t)(n / c) * 4;
         // as many stages as the shared-memory budget holds: a stage is refilled only
         // once every row of it has been used, so the ring is what keeps HBM busy
         const size_t hdr = (8 * kFusedMaxStages + wide_sums_bytes(c) + 127) / 128 * 128;
         int64_t nst = (int64_t)(((size_t)kFusedSmemBudget - hdr) / stage);
         if (nst < 2) nst = 2;
+        if (p->lag && nst < kWideLag + 2) return false;  // the lag's rows + one stage in flight
         if (nst > kFusedMaxStages) nst = kFusedMaxStages;
         if (tune.nst != 0) {
             if (tune.nst < 2 || tune.nst > kFusedMaxStages) return false;
@@ -412,14 +424,15 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
 
 // algo = auto: the single-block kernel from n = 256 up; the cluster kernel only
 // where it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
-// clusters of 8 blocks whose slices are whole multiples of 512 float4, e.g.
-// 8192x32768 259 vs 309 us, 4096x65536 245 vs 323; other shapes lose)
+// clusters of 8 blocks, or the lagged form, with slices that are whole
+// multiples of 512 float4: 8192x32768 259 vs 309 us, 4096x65536 212 vs 322,
+// 1024x131072 157 vs 177; other shapes lose)
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     if (!atax_fused_supported(m, n, aligned16) || n < kFusedMinN) return false;
     FusedPlan p;
     if (fused_plan(n, &p)) return true;
     WidePlan w;
-    return wide_plan(n, &w) && w.clu == 8 && (n / w.clu / 4) % kFusedThreads == 0;
+    return wide_plan(n, &w) && (w.clu == 8 || w.lag) && (n / w.clu / 4) % kFusedThreads == 0;
 }
 
 bool atax_fused_exchange_supported(int64_t m, int64_t n, bool aligned16) {
@@ -1151,10 +1164,139 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     grid_depart(gbar);
 }
 
+// Lagged wide-row kernel (kWideLagged): one row per step; step k computes and
+// pushes the slice dots of row k, then applies the rank-1 update of row k-L
+// (L = kWideLag) once every block's sums of that row are in, re-reading its
+// slice from the ring (rows stay in the ring until their update, then the last
+// warp done refills the slot).  A block therefore waits for its peers L steps
+// late instead of one, which absorbs their data-arrival jitter.  2L+2 sum
+// buffers: a writer at step j has seen every block push row j-1-L, and no
+// reader is further back than row j-1-2L.
+template <int QC, int C>
+__global__ void __launch_bounds__(kFusedThreads, 1)
+    k_atax_fused_wide_lag(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A,
+                          const float *__restrict__ x, float *__restrict__ P, float *__restrict__ y,
+                          unsigned int *__restrict__ gbar, bool discard_partials) {
+    constexpr int L = kWideLag, R = kWideLagBufs;
+    extern __shared__ __align__(128) unsigned char smem[];
+    uint64_t *full = reinterpret_cast<uint64_t *>(smem);
+    uint64_t *sfull = full + kFusedMaxStages;                                  // [R]
+    unsigned int *used = reinterpret_cast<unsigned int *>(sfull + R);         // [16]
+    float *sums = reinterpret_cast<float *>(used + kFusedMaxStages);           // [R][C][16]
+    float *stage0 = reinterpret_cast<float *>(smem + hdr);
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int tid = threadIdx.x;
+    const int r = (int)cluster_ctarank();
+    const int64_t K = cluster_count_x(), kc = cluster_id_x();
+    const int64_t nc = n / C, nvs = nc / 4, col0 = (int64_t)r * nc;
+    const int64_t nstages = kc < m ? (m - kc + K - 1) / K : 0;  // rows kc, kc+K, ...
+    constexpr int SB = C * kFusedWarps;
+    constexpr uint32_t kStepBytes = SB * 4;
+    auto issue_stage = [&](int64_t j, int slot) {
+        mbar_arrive_expect_tx(full + slot, (uint32_t)(nc * 4));
+        bulk_g2s(stage0 + (size_t)slot * nc, A + (j * K + kc) * n + col0, (uint32_t)(nc * 4), full + slot);
+    };
+    if (tid == 0) {
+        for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
+        for (int i = 0; i < R; ++i) mbar_init(sfull + i, 1);
+        for (int i = 0; i < kFusedMaxStages; ++i) used[i] = 0u;
+        fence_mbar_init();
+    }
+    cluster_sync();  // every block's barriers initialised before anyone pushes into it
+    if (tid == 0)
+        for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
+
+    const float4 *x4 = reinterpret_cast<const float4 *>(x + col0);
+    float4 xr[QC], yr[QC];
+#pragma unroll
+    for (int q = 0; q < QC; ++q) {
+        const int64_t c = tid + (int64_t)kFusedThreads * q;
+        xr[q] = c < nvs ? ld_ro4(x4 + c) : zero4();
+        yr[q] = zero4();
+    }
+    int slot = 0, sb = 0, lslot = 0, lsb = 0;
+    uint32_t phase = 0, sphase = 0, lsphase = 0;
+    for (int64_t k = 0; k < nstages + L; ++k) {
+        if (k < nstages) {
+            if (tid == 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);  // arm buffer k % R
+            mbar_wait_parity(full + slot, phase);
+            const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)slot * nc);
+            float4 acc = zero4();
+#pragma unroll
+            for (int q = 0; q < QC; ++q) {
+                const int64_t c = tid + (int64_t)kFusedThreads * q;
+                fma4(acc, c < nvs ? S4[c] : zero4(), xr[q]);
+            }
+            const float dr = warp_sum(hsum4(acc));  // every lane holds the warp's sum
+            const uint32_t la = smem_u32(sums + sb * SB + r * kFusedWarps + warp);
+            const uint32_t lb = smem_u32(sfull + sb);
+#pragma unroll
+            for (int b = 0; b < C; b += 32)
+                if (b + lane < C)
+                    st_async_dsmem1(dsmem_addr_raw(la, (uint32_t)(b + lane)), dr, dsmem_addr_raw(lb, (uint32_t)(b + lane)));
+            if (++slot == nst) {
+                slot = 0;
+                phase ^= 1u;
+            }
+            if (++sb == R) {
+                sb = 0;
+                sphase ^= 1u;
+            }
+        }
+        if (k >= L) {  // the rank-1 update of row k - L
+            mbar_wait_parity(sfull + lsb, lsphase);  // every block's sums of that row
+            // t = pairwise tree over the row's C x 16 sums in (block, warp) order: each
+            // lane's C*16/32 contiguous sums, then a butterfly over the warp
+            constexpr int VPL = SB / 32;
+            float v[VPL];
+            const float *pb = sums + lsb * SB + lane * VPL;
+#pragma unroll
+            for (int u = 0; u < VPL; ++u) v[u] = pb[u];
+            float t = pair_tree<VPL>(v);
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) t = __fadd_rn(t, __shfl_xor_sync(0xffffffffu, t, o));
+            const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)lslot * nc);
+#pragma unroll
+            for (int q = 0; q < QC; ++q) {
+                const int64_t c = tid + (int64_t)kFusedThreads * q;
+                if (c < nvs) fma4s(yr[q], S4[c], t);
+            }
+            // the last of the 16 warps done with the row's slot refills it
+            __syncwarp();
+            if (lane == 0) {
+                if (atom_acq_rel_add_cta_shared(used + lslot, 1u) == kFusedWarps - 1) {
+                    used[lslot] = 0u;
+                    if (k - L + nst < nstages) issue_stage(k - L + nst, lslot);
+                }
+            }
+            if (++lslot == nst) lslot = 0;
+            if (++lsb == R) {
+                lsb = 0;
+                lsphase ^= 1u;
+            }
+        }
+    }
+    cluster_sync();  // no block leaves while a peer's pushes may still land in it
+    float4 *P4 = reinterpret_cast<float4 *>(P + kc * n + col0);
+#pragma unroll
+    for (int q = 0; q < QC; ++q) {
+        const int64_t c = tid + (int64_t)kFusedThreads * q;
+        if (c < nvs) P4[c] = yr[q];
+    }
+    grid_barrier(gbar);
+    const int64_t nv = n / 4;
+    const bool lines = discard_partials;
+    const int64_t unit = lines ? 8 : 1, nu = (nv + unit - 1) / unit;
+    int64_t c0 = unit * (nu * blockIdx.x / gridDim.x), c1 = unit * (nu * (blockIdx.x + 1) / gridDim.x);
+    if (c1 > nv) c1 = nv;
+    colsum_slice<8>((int)K, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0), lines);
+    grid_depart(gbar);
+}
+
 template <int QC, int CR, int C>
 static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, int64_t n, const float *A,
                             const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s) {
-    auto k = k_atax_fused_wide<QC, CR, C>;
+    auto k = CR == 1 ? k_atax_fused_wide_lag<QC, C> : k_atax_fused_wide<QC, CR, C>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
     if (e != cudaSuccess) return e;
@@ -1215,10 +1357,12 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
 #define LIFT_WIDE_PRELOAD(QC, CR, C) \
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<QC, CR, C>);
-    LIFT_WIDE_PRELOAD(1, 4, 2) LIFT_WIDE_PRELOAD(2, 4, 2) LIFT_WIDE_PRELOAD(4, 2, 2)
-    LIFT_WIDE_PRELOAD(1, 4, 4) LIFT_WIDE_PRELOAD(2, 4, 4) LIFT_WIDE_PRELOAD(4, 2, 4)
-    LIFT_WIDE_PRELOAD(1, 4, 8) LIFT_WIDE_PRELOAD(2, 4, 8) LIFT_WIDE_PRELOAD(4, 2, 8)
-    LIFT_WIDE_PRELOAD(1, 4, 16) LIFT_WIDE_PRELOAD(2, 4, 16) LIFT_WIDE_PRELOAD(4, 2, 16)
+    LIFT_WIDE_PRELOAD(1, 4, 2) LIFT_WIDE_PRELOAD(2, 4, 2) LIFT_WIDE_PRELOAD(1, 4, 4) LIFT_WIDE_PRELOAD(2, 4, 4)
+    LIFT_WIDE_PRELOAD(1, 4, 8) LIFT_WIDE_PRELOAD(2, 4, 8) LIFT_WIDE_PRELOAD(1, 4, 16) LIFT_WIDE_PRELOAD(2, 4, 16)
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 8>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 16>);
 #undef LIFT_WIDE_PRELOAD
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<4, 256, 8>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<1, 256, 8>);
@@ -1240,10 +1384,10 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
         float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
 #define LIFT_WIDE_CASE(QC, CR, C) \
     if (w.qc == QC && w.cr == CR && w.clu == C) return run_wide<QC, CR, C>(d, w, m, n, A, x, P, y, gbar, s);
-        LIFT_WIDE_CASE(1, 4, 2) LIFT_WIDE_CASE(2, 4, 2) LIFT_WIDE_CASE(4, 2, 2)
-        LIFT_WIDE_CASE(1, 4, 4) LIFT_WIDE_CASE(2, 4, 4) LIFT_WIDE_CASE(4, 2, 4)
-        LIFT_WIDE_CASE(1, 4, 8) LIFT_WIDE_CASE(2, 4, 8) LIFT_WIDE_CASE(4, 2, 8)
-        LIFT_WIDE_CASE(1, 4, 16) LIFT_WIDE_CASE(2, 4, 16) LIFT_WIDE_CASE(4, 2, 16)
+        LIFT_WIDE_CASE(1, 4, 2) LIFT_WIDE_CASE(2, 4, 2) LIFT_WIDE_CASE(4, 1, 2)
+        LIFT_WIDE_CASE(1, 4, 4) LIFT_WIDE_CASE(2, 4, 4) LIFT_WIDE_CASE(4, 1, 4)
+        LIFT_WIDE_CASE(1, 4, 8) LIFT_WIDE_CASE(2, 4, 8) LIFT_WIDE_CASE(4, 1, 8)
+        LIFT_WIDE_CASE(1, 4, 16) LIFT_WIDE_CASE(2, 4, 16) LIFT_WIDE_CASE(4, 1, 16)
 #undef LIFT_WIDE_CASE
         return cudaErrorInvalidValue;
     }

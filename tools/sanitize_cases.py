@@ -44,7 +44,7 @@ for m, n in ((40, 32), (200, 4096), (300, 8192)):
     for clu in (2, 8):  # thread-block-cluster second stage (DSMEM fold, per-slice tickets)
         chk(f"atax-fused-cluster{clu}-{m}x{n}", lift.lift_atax_fused_tuned(t(A), t(x), cluster=clu).cpu().numpy(),
             *oracle.atax(A, x))
-for m, n in ((9, 20000), (40, 32768)):  # wide rows: the thread-block-cluster single pass
+for m, n in ((9, 20000), (40, 32768), (6, 65536)):  # wide rows: the thread-block-cluster single pass (+ lagged form)
     A = synth.numpy_matrix_rows(2, n, 0, m)
     x = synth.numpy_uniform(0, 0, n)
     chk(f"atax-fused-wide{m}x{n}", lift.lift_atax(t(A), t(x), algo="fused").cpu().numpy(), *oracle.atax(A, x))
