@@ -353,55 +353,40 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
 // fixed-order sum of the C blocks' slice dots.
 // ---------------------------------------------------------------------------
 struct WidePlan {
-    int clu;      // cluster size C (2, 4, 8 or 16)
-    int qc;       // float4 columns per thread within the slice (1, 2 or 4)
-    int cr;       // rows per step (4; 1 in the lagged form)
-    bool lag;     // lagged form (qc = 4)
-    int nst;      // ring stages (cr row slices each)
+    int clu;      // cluster size C (2, 4, 8 or 16); a thread owns 4 float4 columns of its slice
+    int nst;      // ring stages (one row slice each)
     size_t hdr;   // mbarriers + pushed warp sums
     size_t smem;  // dynamic smem bytes
 };
 
-constexpr int kWideRows = 4;  // rows per step (at most)
-constexpr int kWideBufs = 4;  // pushed-sum buffers (a producer is at most 3 steps ahead of a reader)
-// Lagged form (slices of more than 1024 float4, i.e. 32 KiB row slices): one
-// row per step, the rank-1 update of a row applied kWideLag steps after its
-// dot (its slice stays in the ring until then), so a block waits for the
-// peers' sums of row k-L, not k-1; 2L+2 sum buffers.  Narrower slices keep 4
-// rows per step in registers: one-row steps would stream 16 KiB copies.
+// The rank-1 update of a row is applied kWideLag steps after its dot.
 constexpr int kWideLag = 2;
 constexpr int kWideLagBufs = 2 * kWideLag + 2;
 
 static size_t wide_sums_bytes(int c) {
-    const size_t a = 8 * kWideBufs + 4 * kFusedMaxStages + (size_t)kWideBufs * kWideRows * c * kFusedWarps * 4;
-    const size_t b = 8 * kWideLagBufs + 4 * kFusedMaxStages + (size_t)kWideLagBufs * c * kFusedWarps * 4;
-    return a > b ? a : b;
+    return 8 * kWideLagBufs + 4 * kFusedMaxStages + (size_t)kWideLagBufs * c * kFusedWarps * 4;
 }
 
 static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) {
     FusedPlan narrow;
     if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it
     if (tune.l2a > 0 || tune.clu > 1 || tune.clu < 0) return false;     // no L2 prefetch / cluster second stage
-    // clusters of 8 measured fastest (profiles/r01z_atax_wide_cluster_probe.txt: 4 and
-    // 16 lose even with more SMs or narrower slices); other sizes only where 8 cannot
-    // split the row into whole float4 slices of at most 2048 float4
-    int order[4] = {8, 2, 4, 16};
-    for (int c : order) {
+    // the smallest cluster whose slices fit 4 float4 columns per thread: slices of
+    // 1024..2048 float4 (16..32 KiB of a row) on as many SMs as possible
+    // (profiles/r01z_atax_wide_cluster_probe.txt)
+    for (int c = 2; c <= kFusedMaxCluster; c *= 2) {
         if (n % (4 * c) != 0) continue;  // every slice a whole number of float4 columns
         const int64_t nvs = n / c / 4;
         if (nvs > 4 * (int64_t)kFusedThreads) continue;
-        if (c == 2 && n % 16 == 0 && n / 16 <= 4 * (int64_t)kFusedThreads) continue;  // prefer 4 over 2
+        if (nvs <= 2 * (int64_t)kFusedThreads) return false;  // not reached for n > 16384
         p->clu = c;
-        p->qc = nvs <= kFusedThreads ? 1 : (nvs <= 2 * kFusedThreads ? 2 : 4);
-        p->lag = p->qc == 4;
-        p->cr = p->lag ? 1 : kWideRows;
-        const size_t stage = (size_t)p->cr * (size_t)(n / c) * 4;
+        const size_t stage = (size_t)(n / c) * 4;  // one row slice
         // as many stages as the shared-memory budget holds: a stage is refilled only
         // once every row of it has been used, so the ring is what keeps HBM busy
         const size_t hdr = (8 * kFusedMaxStages + wide_sums_bytes(c) + 127) / 128 * 128;
         int64_t nst = (int64_t)(((size_t)kFusedSmemBudget - hdr) / stage);
         if (nst < 2) nst = 2;
-        if (p->lag && nst < kWideLag + 2) return false;  // the lag's rows + one stage in flight
+        if (nst < kWideLag + 2) return false;  // the lagged rows + one stage in flight
         if (nst > kFusedMaxStages) nst = kFusedMaxStages;
         if (tune.nst != 0) {
             if (tune.nst < 2 || tune.nst > kFusedMaxStages) return false;
@@ -422,17 +407,18 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
     return aligned16 && m > 0 && (fused_plan(n, &p) || wide_plan(n, &w));
 }
 
-// algo = auto: the single-block kernel from n = 256 up; the cluster kernel only
-// where it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
-// clusters of 8 blocks, or the lagged form, with slices that are whole
-// multiples of 512 float4: 8192x32768 259 vs 309 us, 4096x65536 212 vs 322,
-// 1024x131072 157 vs 177; other shapes lose)
+// algo = auto: the single-block kernel from n = 256 up; the cluster kernel where
+// it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
+// 8192x32768 174 vs 309 us, 4096x65536 212 vs 322, 8192x20000 176 vs 196) —
+// all but slices barely over 1024 float4 (16384x16416: 339 vs 319), whose
+// threads' fourth column is nearly empty
+constexpr int64_t kWideMinAuto = 1152;
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     if (!atax_fused_supported(m, n, aligned16) || n < kFusedMinN) return false;
     FusedPlan p;
     if (fused_plan(n, &p)) return true;
     WidePlan w;
-    return wide_plan(n, &w) && (w.clu == 8 || w.lag) && (n / w.clu / 4) % kFusedThreads == 0;
+    return wide_plan(n, &w) && n / w.clu / 4 >= kWideMinAuto;
 }
 
 bool atax_fused_exchange_supported(int64_t m, int64_t n, bool aligned16) {
@@ -982,199 +968,25 @@ static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m,
                               rows_are_lines(P, n), clu);
 }
 
-// Wide-row fused ATAX (see WidePlan).  Cluster kc of K streams the row groups
-// (CR consecutive rows) kc, kc+K, ...; its block r reads the groups' column
-// slice r (CR bulk copies per stage into a ring, as k_atax_fused).
-// Step k: the slice dots of group k are reduced per warp and PUSHED into
-// every block's sum buffer k % 4 with asynchronous remote stores
-// (st.async ... mbarrier::complete_tx), each completing bytes on the
-// destination's "sums full" mbarrier of that buffer, which its owner arms with
-// the step's expected bytes.  Then the block waits for buffer (k-1) % 4 to be
-// full (every block's group k-1 sums landed) and applies group k-1's rank-1
-// updates: t_r = pairwise tree over row r's C x 16 sums in (block, warp)
-// order.  No cluster barrier in the loop: blocks drift freely, and a producer
-// can be at most three steps ahead of any reader, so four buffers suffice.
-// No block barrier either: the last warp done with a ring slot refills it.
+// Wide-row fused ATAX (see WidePlan).  Cluster kc of K streams rows kc, kc+K,
+// ...; its block r reads each row's column slice r (one bulk copy per row into
+// a ring).  Step k computes the slice dot of row k, reduces it per warp and
+// PUSHES the warp sums into every block of the cluster with asynchronous remote
+// stores (st.async ... mbarrier::complete_tx), each completing bytes on the
+// destination's "sums full" mbarrier of that buffer, armed by its owner with
+// the step's expected bytes.  Then it applies the rank-1 update of row k-L
+// (L = kWideLag) once every block's sums of that row are in: t = pairwise tree
+// over the row's C x 16 sums in (block, warp) order, and the row's slice is
+// re-read from the ring (a row stays in its slot until its update; the last of
+// the 16 warps done with it refills the slot).  No cluster or block barrier in
+// the loop, and a block waits for its peers L steps late, which absorbs their
+// data-arrival jitter.  2L+2 sum buffers: a writer at step j has seen every
+// block push row j-1-L, and no reader is further back than row j-1-2L.
 // Second stage: partial y rows P[kc][slice] -> grid barrier -> fixed-order
 // column sum over the K cluster rows.
-template <int QC, int CR, int C>
-__global__ void __launch_bounds__(kFusedThreads, 1)
-    k_atax_fused_wide(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A,
-                      const float *__restrict__ x, float *__restrict__ P, float *__restrict__ y,
-                      unsigned int *__restrict__ gbar, bool discard_partials) {
-    extern __shared__ __align__(128) unsigned char smem[];
-    uint64_t *full = reinterpret_cast<uint64_t *>(smem);
-    uint64_t *sfull = full + kFusedMaxStages;                              // [4]
-    unsigned int *used = reinterpret_cast<unsigned int *>(sfull + kWideBufs);  // [16] warps done with a slot
-    float *sums = reinterpret_cast<float *>(used + kFusedMaxStages);       // [4][CR][C][16]
-    float *stage0 = reinterpret_cast<float *>(smem + hdr);
-    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int tid = threadIdx.x;
-    const int r = (int)cluster_ctarank();
-    const int64_t K = cluster_count_x(), kc = cluster_id_x();
-    const int64_t nc = n / C, nvs = nc / 4, col0 = (int64_t)r * nc;
-    const int64_t groups = (m + CR - 1) / CR;
-    const int64_t nstages = kc < groups ? (groups - kc + K - 1) / K : 0;
-    const size_t stage_floats = (size_t)CR * nc;
-    constexpr int SB = CR * C * kFusedWarps;  // floats per sum buffer
-    constexpr uint32_t kStepBytes = SB * 4;   // bytes every block pushes into one buffer per step
-    auto stage_rows = [&](int64_t j) -> int {
-        if (j >= nstages) return 0;
-        const int64_t r0 = (j * K + kc) * CR;
-        return (int)(m - r0 < CR ? m - r0 : CR);
-    };
-    auto issue_stage = [&](int64_t j, int slot) {
-        const int rows = stage_rows(j);
-        const int64_t r0 = (j * K + kc) * CR;
-        mbar_arrive_expect_tx(full + slot, (uint32_t)(rows * nc * 4));
-        for (int i = 0; i < rows; ++i)
-            bulk_g2s(stage0 + (size_t)slot * stage_floats + (size_t)i * nc, A + (r0 + i) * n + col0,
-                     (uint32_t)(nc * 4), full + slot);
-    };
-    if (tid == 0) {
-        for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
-        for (int i = 0; i < kWideBufs; ++i) mbar_init(sfull + i, 1);
-        for (int i = 0; i < kFusedMaxStages; ++i) used[i] = 0u;
-        fence_mbar_init();
-    }
-    // every block's barriers are initialised and it is running before anyone
-    // pushes into its shared memory
-    cluster_sync();
-    if (tid == 0)
-        for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
-
-    const float4 *x4 = reinterpret_cast<const float4 *>(x + col0);
-    float4 xr[QC], yr[QC];
-#pragma unroll
-    for (int q = 0; q < QC; ++q) {
-        const int64_t c = tid + (int64_t)kFusedThreads * q;
-        xr[q] = c < nvs ? ld_ro4(x4 + c) : zero4();
-        yr[q] = zero4();
-    }
-    int sb = 0, psb = 0, slot = 0, pslot = 0, prow = 0;
-    uint32_t phase = 0, sphase = 0, psphase = 0;  // ring parity; sum-buffer parity of steps k and k-1
-    int64_t k = 0;
-    float4 ra[CR][QC], rb2[CR][QC];
-    auto step = [&](float4(&cur)[CR][QC], float4(&prev)[CR][QC]) -> bool {
-        const int rows = stage_rows(k);
-        // no block barrier in the loop: warps of a block are at most one step apart
-        // (a warp at step k has seen every warp's group k-1 push), so warp 0 may arm
-        // buffer k % 4 (last used by step k-4, waited for by every warp by step k-3)
-        if (tid == 0 && rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);
-        if (rows > 0) {
-            mbar_wait_parity(full + slot, phase);
-            const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)slot * stage_floats);
-            float d[CR];
-#pragma unroll
-            for (int i = 0; i < CR; ++i) {
-                float4 acc = zero4();
-#pragma unroll
-                for (int q = 0; q < QC; ++q) {
-                    const int64_t c = tid + (int64_t)kFusedThreads * q;
-                    cur[i][q] = (i < rows && c < nvs) ? S4[(int64_t)i * nvs + c] : zero4();
-                    fma4(acc, cur[i][q], xr[q]);
-                }
-                d[i] = hsum4(acc);
-            }
-            // this warp is done with the ring slot: the last of the 16 warps to get here
-            // refills it with stage k + nst (acq_rel orders every warp's reads before it)
-            __syncwarp();
-            if (lane == 0) {
-                if (atom_acq_rel_add_cta_shared(used + slot, 1u) == kFusedWarps - 1) {
-                    used[slot] = 0u;
-                    if (k + nst < nstages) issue_stage(k + nst, slot);
-                }
-            }
-            // row i's warp sum ends in lanes [i*32/CR, (i+1)*32/CR): lane i*32/CR + b
-            // pushes it to block b (and b + 32/CR, ... when C > 32/CR)
-            const float dr = row_butterfly<CR>(d, lane);
-            const int li = lane & (32 / CR - 1), row = lane / (32 / CR);
-            const uint32_t la = smem_u32(sums + sb * SB + (row * C + r) * kFusedWarps + warp);
-            const uint32_t lb = smem_u32(sfull + sb);
-#pragma unroll
-            for (int b = 0; b < C; b += 32 / CR)
-                if (b + li < C)
-                    st_async_dsmem1(dsmem_addr_raw(la, (uint32_t)(b + li)), dr, dsmem_addr_raw(lb, (uint32_t)(b + li)));
-        }
-        if (prow > 0) {
-            mbar_wait_parity(sfull + psb, psphase);  // every block's group k-1 sums are here
-            // t_r = pairwise tree over row r's C x 16 sums in (block, warp) order (=
-            // a pairwise tree over the blocks of each block's pairwise tree over its
-            // warps).  The CR rows are folded over the warp: 32/CR lanes per row, each
-            // lane's 2C contiguous sums are the lowest tree levels, a butterfly over
-            // the row's lanes the rest; then every lane takes the CR results.
-            constexpr int LPR = 32 / CR, VPL = C * kFusedWarps / LPR;
-            const int row = lane / LPR, li = lane % LPR;
-            const float4 *pb4 = reinterpret_cast<const float4 *>(sums + psb * SB + row * C * kFusedWarps + li * VPL);
-            float v[VPL];
-#pragma unroll
-            for (int u = 0; u < VPL / 4; ++u) {
-                const float4 f = pb4[u];
-                v[4 * u] = f.x;
-                v[4 * u + 1] = f.y;
-                v[4 * u + 2] = f.z;
-                v[4 * u + 3] = f.w;
-            }
-            float tv = pair_tree<VPL>(v);
-#pragma unroll
-            for (int o = 1; o < LPR; o <<= 1) tv = __fadd_rn(tv, __shfl_xor_sync(0xffffffffu, tv, o));
-#pragma unroll
-            for (int i = 0; i < CR; ++i) {
-                const float t = __shfl_sync(0xffffffffu, tv, i * LPR);
-                if (i < prow)
-#pragma unroll
-                    for (int q = 0; q < QC; ++q) fma4s(yr[q], prev[i][q], t);
-            }
-        }
-        if (rows == 0) return true;
-        prow = rows;
-        pslot = slot;
-        if (++slot == nst) {
-            slot = 0;
-            phase ^= 1u;
-        }
-        psb = sb;
-        psphase = sphase;
-        if (++sb == kWideBufs) {
-            sb = 0;
-            sphase ^= 1u;
-        }
-        ++k;
-        return false;
-    };
-    for (;;) {
-        if (step(ra, rb2)) break;
-        if (step(rb2, ra)) break;
-    }
-    cluster_sync();  // no block leaves while a peer's pushes or reads may still involve it
-    // partial y row of this cluster, this block's slice
-    float4 *P4 = reinterpret_cast<float4 *>(P + kc * n + col0);
-#pragma unroll
-    for (int q = 0; q < QC; ++q) {
-        const int64_t c = tid + (int64_t)kFusedThreads * q;
-        if (c < nvs) P4[c] = yr[q];
-    }
-    grid_barrier(gbar);
-    const int64_t nv = n / 4;
-    const bool lines = discard_partials;
-    const int64_t unit = lines ? 8 : 1, nu = (nv + unit - 1) / unit;
-    int64_t c0 = unit * (nu * blockIdx.x / gridDim.x), c1 = unit * (nu * (blockIdx.x + 1) / gridDim.x);
-    if (c1 > nv) c1 = nv;
-    colsum_slice<8>((int)K, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0), lines);
-    grid_depart(gbar);
-}
-
-// Lagged wide-row kernel (kWideLagged): one row per step; step k computes and
-// pushes the slice dots of row k, then applies the rank-1 update of row k-L
-// (L = kWideLag) once every block's sums of that row are in, re-reading its
-// slice from the ring (rows stay in the ring until their update, then the last
-// warp done refills the slot).  A block therefore waits for its peers L steps
-// late instead of one, which absorbs their data-arrival jitter.  2L+2 sum
-// buffers: a writer at step j has seen every block push row j-1-L, and no
-// reader is further back than row j-1-2L.
 template <int QC, int C>
 __global__ void __launch_bounds__(kFusedThreads, 1)
-    k_atax_fused_wide_lag(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A,
+    k_atax_fused_wide(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A,
                           const float *__restrict__ x, float *__restrict__ P, float *__restrict__ y,
                           unsigned int *__restrict__ gbar, bool discard_partials) {
     constexpr int L = kWideLag, R = kWideLagBufs;
@@ -1293,10 +1105,10 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     grid_depart(gbar);
 }
 
-template <int QC, int CR, int C>
+template <int C>
 static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, int64_t n, const float *A,
                             const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s) {
-    auto k = CR == 1 ? k_atax_fused_wide_lag<QC, C> : k_atax_fused_wide<QC, CR, C>;
+    auto k = k_atax_fused_wide<4, C>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
     if (e != cudaSuccess) return e;
@@ -1326,7 +1138,7 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
     {
         std::lock_guard<std::mutex> lock(mu);
         for (int i = 0; i < used; ++i)
-            if (cache[i].dev == d.device && cache[i].clu == C && cache[i].qc == QC && cache[i].nst == p.nst &&
+            if (cache[i].dev == d.device && cache[i].clu == C && cache[i].nst == p.nst &&
                 cache[i].smem == p.smem)
                 nc = cache[i].nc;
         if (nc < 0) {
@@ -1334,14 +1146,13 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
                 (void)cudaGetLastError();
                 nc = 0;
             }
-            if (used < 16) cache[used++] = Entry{d.device, C, QC, p.nst, p.smem, nc};
+            if (used < 16) cache[used++] = Entry{d.device, C, 4, p.nst, p.smem, nc};
         }
     }
     int64_t K = nc;
     if (K < 1) return cudaErrorInvalidConfiguration;
     if (K > kMaxSplits) K = kMaxSplits;
-    const int64_t groups = (m + CR - 1) / CR;
-    if (K > groups) K = groups;
+    if (K > m) K = m;
     cfg.gridDim = dim3((unsigned)(K * C));
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
 }
@@ -1355,19 +1166,10 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
-#define LIFT_WIDE_PRELOAD(QC, CR, C) \
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<QC, CR, C>);
-    LIFT_WIDE_PRELOAD(1, 4, 2) LIFT_WIDE_PRELOAD(2, 4, 2) LIFT_WIDE_PRELOAD(1, 4, 4) LIFT_WIDE_PRELOAD(2, 4, 4)
-    LIFT_WIDE_PRELOAD(1, 4, 8) LIFT_WIDE_PRELOAD(2, 4, 8) LIFT_WIDE_PRELOAD(1, 4, 16) LIFT_WIDE_PRELOAD(2, 4, 16)
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 2>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 4>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 8>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide_lag<4, 16>);
-#undef LIFT_WIDE_PRELOAD
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<4, 256, 8>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_cols<1, 256, 8>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_colsum<4>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_colsum<1>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 8>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 16>);
     return e;
 }
 
@@ -1382,13 +1184,10 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
         if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
         unsigned int *gbar = static_cast<unsigned int *>(ws);
         float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
-#define LIFT_WIDE_CASE(QC, CR, C) \
-    if (w.qc == QC && w.cr == CR && w.clu == C) return run_wide<QC, CR, C>(d, w, m, n, A, x, P, y, gbar, s);
-        LIFT_WIDE_CASE(1, 4, 2) LIFT_WIDE_CASE(2, 4, 2) LIFT_WIDE_CASE(4, 1, 2)
-        LIFT_WIDE_CASE(1, 4, 4) LIFT_WIDE_CASE(2, 4, 4) LIFT_WIDE_CASE(4, 1, 4)
-        LIFT_WIDE_CASE(1, 4, 8) LIFT_WIDE_CASE(2, 4, 8) LIFT_WIDE_CASE(4, 1, 8)
-        LIFT_WIDE_CASE(1, 4, 16) LIFT_WIDE_CASE(2, 4, 16) LIFT_WIDE_CASE(4, 1, 16)
-#undef LIFT_WIDE_CASE
+        if (w.clu == 2) return run_wide<2>(d, w, m, n, A, x, P, y, gbar, s);
+        if (w.clu == 4) return run_wide<4>(d, w, m, n, A, x, P, y, gbar, s);
+        if (w.clu == 8) return run_wide<8>(d, w, m, n, A, x, P, y, gbar, s);
+        if (w.clu == 16) return run_wide<16>(d, w, m, n, A, x, P, y, gbar, s);
         return cudaErrorInvalidValue;
     }
     if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);

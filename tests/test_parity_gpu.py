@@ -330,6 +330,12 @@ def test_gesummv_reductions_bitwise(cuda_device):
 ATAX_SHAPES = [(1, 1), (5, 3), (3, 7), (64, 32), (1000, 300), (300, 1001), (4096, 4096), (2000, 16384), (100, 20000)]
 
 
+def cluster_of(n: int) -> int:
+    """Cluster size the single-pass ATAX uses for wide rows: the smallest C whose
+    column slices are whole float4 columns, at most 2048 float4."""
+    return next(c for c in (2, 4, 8, 16) if n % (4 * c) == 0 and n // c // 4 <= 2048)
+
+
 def fused_supported(n: int) -> bool:
     """Shapes the single-pass ATAX accepts (16-B aligned operands): n % 4 == 0 and
     either n <= 16384 (one block per row) or a cluster of C in {2, 4, 8, 16}
@@ -338,7 +344,12 @@ def fused_supported(n: int) -> bool:
         return False
     if n <= 16384:
         return True
-    return any(n % (4 * c) == 0 and n // c // 4 <= 2048 for c in (2, 4, 8, 16))
+    for c in (2, 4, 8, 16):
+        if n % (4 * c):
+            return False
+        if n // c // 4 <= 2048:
+            return True
+    return False
 
 
 @pytest.mark.parametrize("m,n", ATAX_SHAPES)
@@ -408,7 +419,7 @@ def test_atax_fused_wide(cuda_device, m, n):
         assert torch.equal(lift.lift_atax(A, x, algo="fused"), got)
     auto = lift.lift_atax(A, x)  # the single pass where it beats the two-pass algorithm
     assert_tol(auto.cpu().numpy(), ref, mag, f"atax auto {m}x{n}")
-    if n in (32768, 65536, 49152, 131072):
+    if n // 4 // cluster_of(n) >= 1152:  # slices well over 1024 float4: auto takes the single pass
         assert torch.equal(auto, got)
     assert_tol(lift.lift_atax(A, x, algo="twopass").cpu().numpy(), ref, mag, f"atax twopass {m}x{n}")
 

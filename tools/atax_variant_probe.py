@@ -35,6 +35,8 @@ VARIANTS = {
                    ("                    st_async_dsmem1(dsmem_addr_raw(la, (uint32_t)(b + li)), dr, dsmem_addr_raw(lb, (uint32_t)(b + li)));",
                     "                    if (dr == 1234.5f) sums[0] = dr;"),
                    ("        if (tid == 0 && rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);", "")],
+    # wide-row cluster kernel: clusters of 4 first (n = 32768 -> 32 KiB slices, lagged form, 132 blocks)
+    "wide_c4": [("    int order[4] = {8, 2, 4, 16};", "    int order[4] = {4, 8, 2, 16};")],
     # 16 KiB stages (more, smaller bulk copies; twice the steps)
     "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
 }
