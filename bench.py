@@ -352,6 +352,10 @@ TABLE1 = [
     ("dot_listing1_2^28", "dot_listing1", dict(n=1 << 28), None),
     ("sgemv_t_8192x8192", "sgemv_t", dict(m=8192, n=8192, beta=0.0), None),
     ("sgemv_t_8192x8192_beta", "sgemv_t", dict(m=8192, n=8192, beta=0.5), None),
+    # NEXT-1 beyond one block's ring: rows of 32768 (k_atax_fused_wide, a thread-block cluster
+    # per row group) against the two-pass algorithm on the same 1 GiB matrix
+    ("atax_8192x32768", "atax", dict(m=8192, n=32768), "fused"),
+    ("atax_8192x32768_twopass", "atax", dict(m=8192, n=32768), "twopass"),
 ]
 
 
