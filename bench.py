@@ -722,6 +722,8 @@ def run_ours(args) -> None:
                              "frac_of_spec_peak": round(gbs / spec_peak(), 4),
                              "ncu_dram_pct_of_peak": nc.get("ncu_dram_pct_of_peak"),
                              "ncu_us": nc.get("us")}
+            if op == "atax" and algo == "fused":  # launch shape: the wide kernel's depends on the part's GPCs
+                table1[tname]["grid_blocks"], table1[tname]["cluster"] = lift.lift_atax_fused_grid(shp["m"], shp["n"])
             del g_
 
     kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 1}[op] for _, op, _, _ in WORKLOAD)

@@ -66,6 +66,16 @@ LIFT_API int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const f
                                    int cluster,
                                    lift_stream_t stream);
 
+/* lift_atax_fused_grid: the launch shape of lift_atax's single pass for an
+ * m x n matrix on the current device, without launching anything: *blocks
+ * thread blocks in clusters of *cluster (1 = no cluster: one block per SM,
+ * rows up to 16384 wide; 2..16 = the wide-row kernel, as many clusters as the
+ * device's cluster occupancy allows — the GPC layout of the part decides it).
+ * LIFT_ERR_BAD_SIZE for shapes the single pass does not take (m < 1, n not a
+ * supported width), LIFT_ERR_NULL_PTR for NULL outputs, LIFT_ERR_CUDA when
+ * there is no device. */
+LIFT_API int lift_atax_fused_grid(int64_t m, int64_t n, int *blocks, int *cluster);
+
 #ifdef __cplusplus
 }
 #endif

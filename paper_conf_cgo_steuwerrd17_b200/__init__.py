@@ -20,7 +20,7 @@ from ._lib import (LIFT_ATAX_AUTO, LIFT_ATAX_FUSED, LIFT_ATAX_TWOPASS, LiftError
                    check, lib, library_path)
 
 __all__ = ["lift_dot", "lift_gemv", "lift_gesummv", "lift_atax", "lift_gemv_tuned", "lift_gesummv_tuned",
-           "lift_atax_fused_tuned",
+           "lift_atax_fused_tuned", "lift_atax_fused_grid",
            "lift_partial_dot", "lift_dot_listing1", "lift_sgemv",
            "LiftError", "lib", "library_path", "KERNELS_PER_CALL"]
 
@@ -225,6 +225,16 @@ def lift_atax_fused_tuned(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | 
         check(L.lift_atax_fused_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
                                       nst, l2_ahead, cyclic, cluster, _stream(dev)))
     return out
+
+
+def lift_atax_fused_grid(m: int, n: int) -> tuple[int, int]:
+    """(blocks, cluster size) of lift_atax's single pass for an m x n matrix on the
+    current device (lift_tuning.h); launches nothing."""
+    import ctypes
+
+    b, c = ctypes.c_int(0), ctypes.c_int(0)
+    check(lib().lift_atax_fused_grid(m, n, ctypes.byref(b), ctypes.byref(c)))
+    return b.value, c.value
 
 
 def lift_partial_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None = None,

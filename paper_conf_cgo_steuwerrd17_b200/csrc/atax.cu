@@ -1107,7 +1107,8 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 
 template <int C>
 static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, int64_t n, const float *A,
-                            const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s) {
+                            const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s,
+                            int *grid_out = nullptr /* only report the grid, launch nothing */) {
     auto k = k_atax_fused_wide<4, C>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
@@ -1154,7 +1155,35 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
     if (K > kMaxSplits) K = kMaxSplits;
     if (K > m) K = m;
     cfg.gridDim = dim3((unsigned)(K * C));
+    if (grid_out != nullptr) {
+        *grid_out = (int)(K * C);
+        return cudaSuccess;
+    }
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
+}
+
+// The grid (blocks, cluster size) lift_atax's single pass launches for (m, n)
+// on this device: one block per SM (cooperative) for n <= 16384, else the
+// cluster occupancy of the wide kernel (the GPC layout decides how many
+// clusters fit).  Launches nothing.
+cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *blocks, int *cluster) {
+    FusedPlan p;
+    if (fused_plan(n, &p)) {
+        int64_t G = d.sms;
+        if (G > kMaxSplits) G = kMaxSplits;
+        if (G > m) G = m;
+        if (G < 1) G = 1;
+        *blocks = (int)G;
+        *cluster = 1;
+        return cudaSuccess;
+    }
+    WidePlan w;
+    if (!wide_plan(n, &w) || m < 1) return cudaErrorInvalidValue;
+    *cluster = w.clu;
+    if (w.clu == 2) return run_wide<2>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
+    if (w.clu == 4) return run_wide<4>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
+    if (w.clu == 8) return run_wide<8>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
+    return run_wide<16>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
 }
 
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)

@@ -231,6 +231,15 @@ int lift_atax(int64_t m, int64_t n, const float *A, const float *x, float *y, vo
     return lift_atax_algo_run(LIFT_ATAX_AUTO, m, n, A, x, y, workspace, workspace_bytes, stream);
 }
 
+int lift_atax_fused_grid(int64_t m, int64_t n, int *blocks, int *cluster) {
+    if (blocks == nullptr || cluster == nullptr) return LIFT_ERR_NULL_PTR;
+    if (!size_ok(m, n) || !lift::atax_fused_supported(m, n, true)) return LIFT_ERR_BAD_SIZE;
+    DeviceInfo d;
+    cudaError_t e = lift::device_info(&d);
+    if (e != cudaSuccess) return cuda_status(e);
+    return cuda_status(lift::atax_fused_grid(d, m, n, blocks, cluster));
+}
+
 int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
                           size_t workspace_bytes, int nst, int l2_ahead, int cyclic, int cluster,
                           lift_stream_t stream) {

@@ -69,6 +69,7 @@ size_t atax_fused_ws_bytes(int64_t m, int64_t n);
 bool atax_fused_supported(int64_t m, int64_t n, bool aligned16);
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16);
 bool atax_fused_exchange_supported(int64_t m, int64_t n, bool aligned16);  // the NVLink-fused form (n <= 16384)
+cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *blocks, int *cluster);
 cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
                                 float *y, void *ws, cudaStream_t s);
 // y = alpha * A^T x + beta * y  (A m x n row-major with stride lda; x in R^m, y in R^n):

@@ -119,6 +119,18 @@ def test_tuned_validation():
     assert L.lift_atax_fused_tuned(64, 512, A_, X_, A_, W_, ws, 0, -1, -1, 0, None) == ALIAS
 
 
+def test_atax_fused_grid_validation():
+    import ctypes
+
+    b, c = ctypes.c_int(0), ctypes.c_int(0)
+    assert L.lift_atax_fused_grid(64, 512, None, ctypes.byref(c)) == NULL
+    assert L.lift_atax_fused_grid(0, 512, ctypes.byref(b), ctypes.byref(c)) == SIZE  # no rows: no launch shape
+    assert L.lift_atax_fused_grid(64, 510, ctypes.byref(b), ctypes.byref(c)) == SIZE  # n % 4
+    assert L.lift_atax_fused_grid(64, 16392, ctypes.byref(b), ctypes.byref(c)) == SIZE  # no whole-float4 slices
+    if not _gpu():
+        assert L.lift_atax_fused_grid(64, 512, ctypes.byref(b), ctypes.byref(c)) == CUDA
+
+
 # ---------------------------------------------------------------- ATAX
 def test_atax_validation():
     m, n = 64, 32

@@ -424,6 +424,19 @@ def test_atax_fused_wide(cuda_device, m, n):
     assert_tol(lift.lift_atax(A, x, algo="twopass").cpu().numpy(), ref, mag, f"atax twopass {m}x{n}")
 
 
+def test_atax_fused_grid(cuda_device):
+    """lift_atax_fused_grid reports the single pass's launch shape: one block per SM
+    up to 16384 columns, whole clusters of the wide kernel beyond (at most one
+    block per SM), and the wide kernel's cluster is the one its slices need."""
+    sms = torch.cuda.get_device_properties(cuda_device).multi_processor_count
+    assert lift.lift_atax_fused_grid(8192, 8192) == (min(sms, 256), 1)
+    assert lift.lift_atax_fused_grid(5, 4096) == (5, 1)
+    for n in (20000, 32768, 65536, 131072):
+        blocks, c = lift.lift_atax_fused_grid(8192, n)
+        assert c == cluster_of(n) and blocks % c == 0 and 0 < blocks <= sms, (n, blocks, c)
+    assert lift.lift_atax_fused_grid(3, 32768) == (3 * 4, 4)  # one cluster per row
+
+
 def test_atax_fused_wide_rejects(cuda_device):
     """Wide rows whose cluster slices would not be whole float4 columns stay on
     the two-pass algorithm (auto) and are refused by algo="fused"."""

@@ -19,6 +19,8 @@ SHAPES = ((2048, 32768), (8192, 32768), (4096, 65536), (8192, 49152), (8192, 245
           (1024, 131072))
 if os.environ.get("WIDE_QUICK"):
     SHAPES = ((8192, 32768), (4096, 65536))
+if os.environ.get("WIDE_SHAPES"):  # e.g. "8192x16384,16384x16384"
+    SHAPES = tuple(tuple(int(v) for v in s.split("x")) for s in os.environ["WIDE_SHAPES"].split(","))
 for m, n in SHAPES:
     sets = max(2, -(-2 * L2 // (4 * m * n)))
     As = [synth.torch_matrix_rows(2 + 10 * k, n, 0, m, device=dev) for k in range(sets)]

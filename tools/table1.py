@@ -31,6 +31,8 @@ for name, op, shp, algo, calls in sets:
             calls[j % len(calls)]()
         torch.cuda.synchronize()
         break
+    if os.environ.get("TABLE1_ONLY") and name not in os.environ["TABLE1_ONLY"].split(","):
+        continue
     from sweep import graph_time  # noqa: E402
 
     reps = max(20, len(calls))
