@@ -37,6 +37,11 @@ VARIANTS = {
                    ("        if (tid == 0 && rows > 0) mbar_arrive_expect_tx(sfull + sb, kStepBytes);", "")],
     # wide-row cluster kernel: clusters of 4 first (n = 32768 -> 32 KiB slices, lagged form, 132 blocks)
     "wide_c4": [("    int order[4] = {8, 2, 4, 16};", "    int order[4] = {4, 8, 2, 16};")],
+    # the cluster kernel also for 8192 < n <= 16384 (C = 2 slices of up to 2048 float4), instead of
+    # the single-block kernel (timing only: tools/atax_wide_probe.py with WIDE_SHAPES)
+    "wide_mid": [("    if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it",
+                  "    if (n <= 0 || n % 4 != 0 || n <= 8192) return false;"),
+                 ("    if (!fused_plan(n, &p, tune)) {", "    WidePlan w0;\n    if (!fused_plan(n, &p, tune) || (n > 8192 && wide_plan(n, &w0, tune))) {")],
     # 16 KiB stages (more, smaller bulk copies; twice the steps)
     "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
 }
