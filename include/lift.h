@@ -131,8 +131,8 @@ LIFT_API int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, flo
  *                      per-block y_part (reads A once: 4*m*n bytes).
  *                      Needs 16-byte aligned A, x, y and n % 4 == 0; rows
  *                      of n <= 16384 are streamed by one block each, wider
- *                      rows (n <= 131072, n a multiple of 4C whose slices
- *                      are at most 2048 float4) by a thread-block cluster
+ *                      rows (n <= 262144, n a multiple of 4C whose slices
+ *                      are at most 4096 float4) by a thread-block cluster
  *                      of C = 2..16 blocks over column slices.  Other
  *                      shapes: LIFT_ERR_BAD_SIZE (auto uses TWOPASS).
  *   LIFT_ATAX_TWOPASS  the paper's structure (two GEMV-shaped kernels whose

@@ -353,15 +353,17 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
 // fixed-order sum of the C blocks' slice dots.
 // ---------------------------------------------------------------------------
 struct WidePlan {
-    int clu;      // cluster size C (2, 4, 8 or 16); a thread owns 4 float4 columns of its slice
+    int clu;      // cluster size C (2, 4, 8 or 16); a thread owns kWideQc float4 columns of its slice
     int nst;      // ring stages (one row slice each)
     size_t hdr;   // mbarriers + pushed warp sums
     size_t smem;  // dynamic smem bytes
 };
 
-// The rank-1 update of a row is applied kWideLag steps after its dot.
-constexpr int kWideLag = 2;
+// The rank-1 update of a row is applied kWideLag steps after its dot; a thread
+// owns kWideQc float4 columns of its block's slice (slices of 2049..4096 float4).
+constexpr int kWideLag = 1;
 constexpr int kWideLagBufs = 2 * kWideLag + 2;
+constexpr int kWideQc = 8;
 
 static size_t wide_sums_bytes(int c) {
     return 8 * kWideLagBufs + 4 * kFusedMaxStages + (size_t)kWideLagBufs * c * kFusedWarps * 4;
@@ -371,14 +373,14 @@ static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) 
     FusedPlan narrow;
     if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it
     if (tune.l2a > 0 || tune.clu > 1 || tune.clu < 0) return false;     // no L2 prefetch / cluster second stage
-    // the smallest cluster whose slices fit 4 float4 columns per thread: slices of
-    // 1024..2048 float4 (16..32 KiB of a row) on as many SMs as possible
-    // (profiles/r01z_atax_wide_cluster_probe.txt)
+    // the smallest cluster whose slices fit kWideQc float4 columns per thread: slices
+    // of 2049..4096 float4 (32..64 KiB of a row) on as many SMs as possible — clusters
+    // of 2 fill all 148 SMs (profiles/r01z_atax_wide_cluster_probe.txt)
     for (int c = 2; c <= kFusedMaxCluster; c *= 2) {
         if (n % (4 * c) != 0) continue;  // every slice a whole number of float4 columns
         const int64_t nvs = n / c / 4;
-        if (nvs > 4 * (int64_t)kFusedThreads) continue;
-        if (nvs <= 2 * (int64_t)kFusedThreads) return false;  // not reached for n > 16384
+        if (nvs > kWideQc * (int64_t)kFusedThreads) continue;
+        if (nvs <= 4 * (int64_t)kFusedThreads) return false;  // not reached for n > 16384
         p->clu = c;
         const size_t stage = (size_t)(n / c) * 4;  // one row slice
         // as many stages as the shared-memory budget holds: a stage is refilled only
@@ -407,18 +409,15 @@ bool atax_fused_supported(int64_t m, int64_t n, bool aligned16) {
     return aligned16 && m > 0 && (fused_plan(n, &p) || wide_plan(n, &w));
 }
 
-// algo = auto: the single-block kernel from n = 256 up; the cluster kernel where
-// it beats the two-pass algorithm (profiles/r01z_atax_wide_cluster_probe.txt:
-// 8192x32768 174 vs 309 us, 4096x65536 212 vs 322, 8192x20000 176 vs 196) —
-// all but slices barely over 1024 float4 (16384x16416: 339 vs 319), whose
-// threads' fourth column is nearly empty
-constexpr int64_t kWideMinAuto = 1152;
+// algo = auto: the single-block kernel from n = 256 up, the cluster kernel for
+// every wider supported row — it beats the two-pass algorithm at every shape
+// measured (profiles/r01z_atax_wide_cluster_probe.txt: 1.6-2.0x)
 bool atax_fused_preferred(int64_t m, int64_t n, bool aligned16) {
     if (!atax_fused_supported(m, n, aligned16) || n < kFusedMinN) return false;
     FusedPlan p;
     if (fused_plan(n, &p)) return true;
     WidePlan w;
-    return wide_plan(n, &w) && n / w.clu / 4 >= kWideMinAuto;
+    return wide_plan(n, &w);
 }
 
 bool atax_fused_exchange_supported(int64_t m, int64_t n, bool aligned16) {
@@ -1109,7 +1108,7 @@ template <int C>
 static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, int64_t n, const float *A,
                             const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s,
                             int *grid_out = nullptr /* only report the grid, launch nothing */) {
-    auto k = k_atax_fused_wide<4, C>;
+    auto k = k_atax_fused_wide<kWideQc, C>;
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
     if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
     if (e != cudaSuccess) return e;
@@ -1195,7 +1194,10 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 2>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 4>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 8>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 16>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 4>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 8>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 16>);

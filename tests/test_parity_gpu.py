@@ -332,8 +332,8 @@ ATAX_SHAPES = [(1, 1), (5, 3), (3, 7), (64, 32), (1000, 300), (300, 1001), (4096
 
 def cluster_of(n: int) -> int:
     """Cluster size the single-pass ATAX uses for wide rows: the smallest C whose
-    column slices are whole float4 columns, at most 2048 float4."""
-    return next(c for c in (2, 4, 8, 16) if n % (4 * c) == 0 and n // c // 4 <= 2048)
+    column slices are whole float4 columns, at most 4096 float4."""
+    return next(c for c in (2, 4, 8, 16) if n % (4 * c) == 0 and n // c // 4 <= 4096)
 
 
 def fused_supported(n: int) -> bool:
@@ -347,7 +347,7 @@ def fused_supported(n: int) -> bool:
     for c in (2, 4, 8, 16):
         if n % (4 * c):
             return False
-        if n // c // 4 <= 2048:
+        if n // c // 4 <= 4096:
             return True
     return False
 
@@ -397,7 +397,7 @@ def test_atax_fused_tuning(cuda_device):
                 lift.lift_atax_fused_tuned(A, x, **bad)
 
 
-WIDE_SHAPES = [(1, 16416), (3, 20000), (300, 32768), (1001, 24576), (64, 65536), (777, 16416), (2048, 32768),
+WIDE_SHAPES = [(1, 16416), (7, 16392), (3, 20000), (300, 32768), (1001, 24576), (64, 65536), (777, 16416), (2048, 32768),
                (9, 16400), (5, 131072), (130, 49152)]
 
 
@@ -419,8 +419,7 @@ def test_atax_fused_wide(cuda_device, m, n):
         assert torch.equal(lift.lift_atax(A, x, algo="fused"), got)
     auto = lift.lift_atax(A, x)  # the single pass where it beats the two-pass algorithm
     assert_tol(auto.cpu().numpy(), ref, mag, f"atax auto {m}x{n}")
-    if n // 4 // cluster_of(n) >= 1152:  # slices well over 1024 float4: auto takes the single pass
-        assert torch.equal(auto, got)
+    assert torch.equal(auto, got)  # auto takes the single pass for every supported wide row
     assert_tol(lift.lift_atax(A, x, algo="twopass").cpu().numpy(), ref, mag, f"atax twopass {m}x{n}")
 
 
@@ -434,13 +433,14 @@ def test_atax_fused_grid(cuda_device):
     for n in (20000, 32768, 65536, 131072):
         blocks, c = lift.lift_atax_fused_grid(8192, n)
         assert c == cluster_of(n) and blocks % c == 0 and 0 < blocks <= sms, (n, blocks, c)
-    assert lift.lift_atax_fused_grid(3, 32768) == (3 * 4, 4)  # one cluster per row
+    c = cluster_of(32768)
+    assert lift.lift_atax_fused_grid(3, 32768) == (3 * c, c)  # one cluster per row
 
 
 def test_atax_fused_wide_rejects(cuda_device):
     """Wide rows whose cluster slices would not be whole float4 columns stay on
     the two-pass algorithm (auto) and are refused by algo="fused"."""
-    for n in (16392, 16388, 20004):
+    for n in (16388, 20004, 32772):
         assert not fused_supported(n)
         A = synth.torch_matrix_rows(synth.SEED_A, n, 0, 5, device=cuda_device)
         x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
