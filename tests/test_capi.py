@@ -126,7 +126,7 @@ def test_atax_fused_grid_validation():
     assert L.lift_atax_fused_grid(64, 512, None, ctypes.byref(c)) == NULL
     assert L.lift_atax_fused_grid(0, 512, ctypes.byref(b), ctypes.byref(c)) == SIZE  # no rows: no launch shape
     assert L.lift_atax_fused_grid(64, 510, ctypes.byref(b), ctypes.byref(c)) == SIZE  # n % 4
-    assert L.lift_atax_fused_grid(64, 16392, ctypes.byref(b), ctypes.byref(c)) == SIZE  # no whole-float4 slices
+    assert L.lift_atax_fused_grid(64, 16388, ctypes.byref(b), ctypes.byref(c)) == SIZE  # no whole-float4 slices
     if not _gpu():
         assert L.lift_atax_fused_grid(64, 512, ctypes.byref(b), ctypes.byref(c)) == CUDA
 
