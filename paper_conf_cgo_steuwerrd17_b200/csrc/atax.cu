@@ -26,6 +26,12 @@
 // The per-block y partials are summed in a fixed order in the SAME launch: a
 // grid barrier (cooperative launch, one block per SM) and then every block
 // reduces a tile of columns over all partial rows.
+//
+// FUSED, WIDE ROWS (n > 16384, k_atax_fused_wide): the columns split over a
+// thread-block cluster; each block streams its column slice of the cluster's
+// rows, the warps' slice dots are pushed into every block of the cluster by
+// asynchronous remote stores (st.async + mbarrier complete_tx), and each row's
+// rank-1 update is applied one row later from the ring.  Same second stage.
 #include <mutex>
 #include <type_traits>
 
