@@ -23,7 +23,8 @@ def test_compute_sanitizer(cuda_device, tool):
     filt = [] if tool == "initcheck" else ["--kernel-name", "kns=lift"]
     cmd = [cs, "--tool", tool, "--error-exitcode", "99", *filt,
            sys.executable, os.path.join(ROOT, "tools", "sanitize_cases.py")]
-    r = subprocess.run(cmd, capture_output=True, text=True, timeout=900, cwd=ROOT)
+    env = dict(os.environ, LIFT_SANITIZER_TOOL=tool)  # tools/sanitize_cases.py: see the wide-row cases
+    r = subprocess.run(cmd, capture_output=True, text=True, timeout=900, cwd=ROOT, env=env)
     tail = (r.stdout + r.stderr)[-4000:]
     assert r.returncode == 0, tail
     assert "sanitize cases ok" in r.stdout, tail
