@@ -370,6 +370,11 @@ struct WidePlan {
 constexpr int kWideLag = 1;
 constexpr int kWideLagBufs = 2 * kWideLag + 2;
 constexpr int kWideQc = 8;
+// Rows wider than this take the wide kernel (clusters of 1 up to 16384: no
+// cluster, x in registers, rows one step late from the ring — 8192x12288 65.7
+// against 72.7 us for the single-block kernel, equal at 16384;
+// profiles/r01zd_atax_wide_c1.txt)
+constexpr int64_t kWideMinN = 8192;
 
 static size_t wide_sums_bytes(int c) {
     return 8 * kWideLagBufs + 4 * kFusedMaxStages + (size_t)kWideLagBufs * c * kFusedWarps * 4;
@@ -377,16 +382,17 @@ static size_t wide_sums_bytes(int c) {
 
 static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) {
     FusedPlan narrow;
-    if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it
+    (void)narrow;
+    if (n <= kWideMinN || n % 4 != 0) return false;  // below: the single-block kernel
     if (tune.l2a > 0 || tune.clu > 1 || tune.clu < 0) return false;     // no L2 prefetch / cluster second stage
     // the smallest cluster whose slices fit kWideQc float4 columns per thread: slices
     // of 2049..4096 float4 (32..64 KiB of a row) on as many SMs as possible — clusters
     // of 2 fill all 148 SMs (profiles/r01z_atax_wide_cluster_probe.txt)
-    for (int c = 2; c <= kFusedMaxCluster; c *= 2) {
+    for (int c = 1; c <= kFusedMaxCluster; c *= 2) {
         if (n % (4 * c) != 0) continue;  // every slice a whole number of float4 columns
         const int64_t nvs = n / c / 4;
         if (nvs > kWideQc * (int64_t)kFusedThreads) continue;
-        if (nvs <= 4 * (int64_t)kFusedThreads) return false;  // not reached for n > 16384
+        if (nvs <= 4 * (int64_t)kFusedThreads) return false;  // not reached for n > kWideMinN
         p->clu = c;
         const size_t stage = (size_t)(n / c) * 4;  // one row slice
         // as many stages as the shared-memory budget holds: a stage is refilled only
@@ -1064,11 +1070,11 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
             mbar_wait_parity(sfull + lsb, lsphase);  // every block's sums of that row
             // t = pairwise tree over the row's C x 16 sums in (block, warp) order: each
             // lane's C*16/32 contiguous sums, then a butterfly over the warp
-            constexpr int VPL = SB / 32;
+            constexpr int VPL = SB >= 32 ? SB / 32 : 1;  // C = 1: lanes 16..31 add zeros
             float v[VPL];
             const float *pb = sums + lsb * SB + lane * VPL;
 #pragma unroll
-            for (int u = 0; u < VPL; ++u) v[u] = pb[u];
+            for (int u = 0; u < VPL; ++u) v[u] = (lane * VPL + u < SB) ? pb[u] : 0.f;
             float t = pair_tree<VPL>(v);
 #pragma unroll
             for (int o = 1; o < 32; o <<= 1) t = __fadd_rn(t, __shfl_xor_sync(0xffffffffu, t, o));
@@ -1173,7 +1179,8 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
 // clusters fit).  Launches nothing.
 cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *blocks, int *cluster) {
     FusedPlan p;
-    if (fused_plan(n, &p)) {
+    WidePlan w0;
+    if (fused_plan(n, &p) && !wide_plan(n, &w0)) {
         int64_t G = d.sms;
         if (G > kMaxSplits) G = kMaxSplits;
         if (G > m) G = m;
@@ -1185,6 +1192,7 @@ cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *bloc
     WidePlan w;
     if (!wide_plan(n, &w) || m < 1) return cudaErrorInvalidValue;
     *cluster = w.clu;
+    if (w.clu == 1) return run_wide<1>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     if (w.clu == 2) return run_wide<2>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     if (w.clu == 4) return run_wide<4>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     if (w.clu == 8) return run_wide<8>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
@@ -1200,6 +1208,7 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 2>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 4>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 8>);
@@ -1214,19 +1223,25 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
                               void *ws, cudaStream_t s, Exch ex, int dst, int blocks, FusedTuning tune) {
     if (n == 0) return cudaSuccess;
     FusedPlan p;
-    if (!fused_plan(n, &p, tune)) {
-        // wide rows: the cluster kernel (single rank, grid from the cluster occupancy)
-        WidePlan w;
-        if (ex.world != 0 || blocks > 0 || !wide_plan(n, &w, tune)) return cudaErrorInvalidValue;
+    // wide rows: the cluster kernel (single rank, default tuning, grid from the
+    // cluster occupancy); explicit tuning and the fused exchanges keep the
+    // single-block kernel where it exists
+    const bool tuned = tune.nst != 0 || tune.l2a > 0 || tune.cyc >= 0 || tune.clu > 1;
+    FusedPlan pdef;
+    const bool narrow_exists = fused_plan(n, &pdef);  // a single-block kernel for this width
+    WidePlan w;
+    if (ex.world == 0 && blocks <= 0 && (!narrow_exists || !tuned) && wide_plan(n, &w, tune)) {
         if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
         unsigned int *gbar = static_cast<unsigned int *>(ws);
         float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
+        if (w.clu == 1) return run_wide<1>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 2) return run_wide<2>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 4) return run_wide<4>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 8) return run_wide<8>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 16) return run_wide<16>(d, w, m, n, A, x, P, y, gbar, s);
         return cudaErrorInvalidValue;
     }
+    if (!fused_plan(n, &p, tune)) return cudaErrorInvalidValue;
     if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
     unsigned int *gbar = static_cast<unsigned int *>(ws);
     float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);

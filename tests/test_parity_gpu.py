@@ -391,7 +391,7 @@ def test_atax_fused_tuning(cuda_device):
                         assert n > 8192 and nst >= 3, (m, n, nst)  # 64 KiB rows + x in smem: 2 stages max
                         continue
                     assert torch.equal(got, base), (m, n, cyc, nst, l2a)
-        assert hits >= 1
+        assert hits >= 1 or n > 8192  # rows wider than 8192: the automatic call takes the wide kernel
         for bad in (dict(nst=1), dict(nst=17), dict(l2_ahead=65), dict(cyclic=2)):
             with pytest.raises(lift.LiftError):
                 lift.lift_atax_fused_tuned(A, x, **bad)

@@ -42,6 +42,18 @@ VARIANTS = {
     "wide_mid": [("    if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it",
                   "    if (n <= 0 || n % 4 != 0 || n <= 8192) return false;"),
                  ("    if (!fused_plan(n, &p, tune)) {", "    WidePlan w0;\n    if (!fused_plan(n, &p, tune) || (n > 8192 && wide_plan(n, &w0, tune))) {")],
+    # the wide kernel without a cluster (C = 1) for 8192 < n <= 16384 instead of the single-block
+    # kernel: x, y in registers, rows re-read from the ring one step late
+    "wide_c1": [("    if (n <= 0 || n % 4 != 0 || fused_plan(n, &narrow)) return false;  // the single-block kernel covers it",
+                 "    if (n <= 0 || n % 4 != 0 || n <= 8192) return false;"),
+                ("    for (int c = 2; c <= kFusedMaxCluster; c *= 2) {\n        if (n % (4 * c) != 0) continue;  // every slice",
+                 "    for (int c = 1; c <= kFusedMaxCluster; c *= 2) {\n        if (n % (4 * c) != 0) continue;  // every slice"),
+                ("    if (!fused_plan(n, &p, tune)) {", "    WidePlan w0;\n    if (!fused_plan(n, &p, tune) || (n > 8192 && wide_plan(n, &w0, tune))) {"),
+                ("        if (w.clu == 2) return run_wide<2>(d, w, m, n, A, x, P, y, gbar, s);",
+                 "        if (w.clu == 1) return run_wide<1>(d, w, m, n, A, x, P, y, gbar, s);\n        if (w.clu == 2) return run_wide<2>(d, w, m, n, A, x, P, y, gbar, s);"),
+                ("            constexpr int VPL = SB / 32;", "            constexpr int VPL = SB >= 32 ? SB / 32 : 1;"),
+                ("            for (int u = 0; u < VPL; ++u) v[u] = pb[u];",
+                 "            for (int u = 0; u < VPL; ++u) v[u] = (lane * VPL + u < SB) ? pb[u] : 0.f;")],
     # 16 KiB stages (more, smaller bulk copies; twice the steps)
     "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
 }
