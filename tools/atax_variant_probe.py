@@ -54,6 +54,10 @@ VARIANTS = {
                 ("            constexpr int VPL = SB / 32;", "            constexpr int VPL = SB >= 32 ? SB / 32 : 1;"),
                 ("            for (int u = 0; u < VPL; ++u) v[u] = pb[u];",
                  "            for (int u = 0; u < VPL; ++u) v[u] = (lane * VPL + u < SB) ? pb[u] : 0.f;")],
+    # the no-cluster wide kernel down to n > 4096 (8192: threads own 4 of their 8 float4 columns)
+    "wide_c1_8k": [("constexpr int64_t kWideMinN = 8192;", "constexpr int64_t kWideMinN = 4096;"),
+                   ("        if (nvs <= 4 * (int64_t)kFusedThreads) return false;  // not reached for n > kWideMinN",
+                    "        if (nvs <= 2 * (int64_t)kFusedThreads) return false;")],
     # 16 KiB stages (more, smaller bulk copies; twice the steps)
     "stage16": [("constexpr size_t kFusedStageTarget = 32 * 1024;", "constexpr size_t kFusedStageTarget = 16 * 1024;")],
 }
