@@ -42,7 +42,9 @@ _lib = None
 def _load():
     global _lib
     if _lib is None:
-        lib = ctypes.CDLL(build())
+        # LIFT_ORACLE_SO: a deliberately mutated copy built by tools/mutate_oracle.py
+        # (mutation testing of the pins); never set otherwise
+        lib = ctypes.CDLL(os.environ.get("LIFT_ORACLE_SO") or build())
         f32p = ctypes.POINTER(ctypes.c_float)
         f64p = ctypes.POINTER(ctypes.c_double)
         i64 = ctypes.c_int64

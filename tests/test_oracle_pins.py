@@ -342,6 +342,9 @@ def test_partial_dot_sums_to_dot_and_drops_tail():
     for k in range(7):
         exact = sum((F(a) * F(b) for a, b in zip(x[128 * k:128 * k + 128], y[128 * k:128 * k + 128])), Fraction(0))
         assert_close_exact([z[k]], [exact], 128, [mag[k]])
+        exact_mag = sum((abs(F(a) * F(b)) for a, b in zip(x[128 * k:128 * k + 128], y[128 * k:128 * k + 128])),
+                        Fraction(0))
+        assert_close_exact([mag[k]], [exact_mag], 128, [mag[k]])
 
 
 @pytest.mark.parametrize("use_fma", [True, False])
@@ -473,6 +476,10 @@ def test_sgemv_bruteforce_fraction(layout, trans, alpha, beta):
     exact = [a32 * s + (b32 * F(yv) if beta != 0 else 0) for s, yv in zip(exact_matvec(opA, x), yin)]
     assert np.all(np.isfinite(y))  # the NaN padding is never read
     assert_close_exact(y, exact, opA.shape[1] + 2, mag)
+    # mag = |alpha| sum_k |op(A)_ok x_k| (+ |beta y_o| when beta != 0), exactly the sum of |terms|
+    exact_mag = [abs(a32) * s + (abs(b32 * F(yv)) if beta != 0 else 0)
+                 for s, yv in zip(exact_abs_matvec(opA, x), yin)]
+    assert_close_exact(mag, exact_mag, opA.shape[1] + 2, mag)
 
 
 def test_sgemv_reduces_to_gemv_and_ignores_y_when_beta_zero():
