@@ -14,11 +14,17 @@
  * is rank r's exchange area as mapped in the calling process (entry `rank` is
  * the caller's own).  One exchange area serves one op at a time.
  *
- * `epoch` numbers the calls made on an exchange area: 1, 2, 3, ... in the same
- * order on every rank (the library never resets flags; data is double
- * buffered by epoch parity, so a rank may run at most one call ahead).
- * Every rank must make the matching call, or the waiting ranks trap after
- * about a minute (cudaErrorLaunchFailure) instead of hanging.
+ * Calls on one exchange area must be made in the same order on every rank
+ * (every rank makes the matching call).  The call counter (epoch) lives in
+ * the area on the device — the host passes none — so a sequence of these
+ * calls can be captured in a CUDA graph and replayed.  Data is double
+ * buffered by epoch parity; before a rank stores into a peer's buffer it
+ * waits (on the device) until that peer has acknowledged consuming the
+ * call two epochs back, so no rank overwrites data a slower rank is still
+ * reading, in any mix of all-reduce, all-gather and reduce-to-one-rank calls.
+ * A rank that never makes the matching call makes its peers trap after the
+ * spin limit (LIFT_SPIN_TIMEOUT_MS, default 20 s; the launch fails with a
+ * CUDA error at the next synchronisation) instead of hanging the GPU.
  *
  * Validation follows lift.h (status codes, nothing enqueued on error); the
  * contents of `peers` live in device memory and are not checked.
@@ -44,7 +50,7 @@ LIFT_API size_t lift_exchange_bytes(int kind, int64_t len, int world);
  * in rank order, identical on every rank.  workspace as in lift_dot.      */
 LIFT_API int lift_dot_allreduce(int64_t n, const float *x, const float *y, float *result,
                                 void *workspace, size_t workspace_bytes,
-                                void *const *peers, int rank, int world, uint64_t epoch,
+                                void *const *peers, int rank, int world,
                                 lift_stream_t stream);
 
 /* GEMV / GESUMMV over row blocks: rank `rank` holds rows [row0, row0+m) of
@@ -55,12 +61,12 @@ LIFT_API int lift_dot_allreduce(int64_t n, const float *x, const float *y, float
 LIFT_API int lift_gemv_allgather(int64_t m, int64_t n, const float *A, const float *x,
                                  int64_t row0, int64_t m_total, float *y,
                                  void *workspace, size_t workspace_bytes,
-                                 void *const *peers, int rank, int world, uint64_t epoch,
+                                 void *const *peers, int rank, int world,
                                  lift_stream_t stream);
 LIFT_API int lift_gesummv_allgather(int64_t m, int64_t n, float alpha, const float *A, float beta,
                                     const float *B, const float *x, int64_t row0, int64_t m_total,
                                     float *y, void *workspace, size_t workspace_bytes,
-                                    void *const *peers, int rank, int world, uint64_t epoch,
+                                    void *const *peers, int rank, int world,
                                     lift_stream_t stream);
 
 /* ATAX over row blocks: y = sum over ranks of A_r^T (A_r x) on rank `dst`
@@ -72,7 +78,7 @@ LIFT_API int lift_gesummv_allgather(int64_t m, int64_t n, float alpha, const flo
  * one GPU in tests: the caller guarantees co-residency).                  */
 LIFT_API int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float *y,
                               void *workspace, size_t workspace_bytes,
-                              void *const *peers, int rank, int world, int dst, uint64_t epoch,
+                              void *const *peers, int rank, int world, int dst,
                               int blocks, lift_stream_t stream);
 
 #ifdef __cplusplus

@@ -50,10 +50,10 @@ SIGNATURES = {
     "lift_dot_listing1_workspace_bytes": (sz, [i64]),
     "lift_dot_listing1": (i32, [i64, vp, vp, vp, vp, sz, i32, vp]),
     "lift_exchange_bytes": (sz, [i32, i64, i32]),
-    "lift_dot_allreduce": (i32, [i64, vp, vp, vp, vp, sz, vp, i32, i32, u64, vp]),
-    "lift_gemv_allgather": (i32, [i64, i64, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, u64, vp]),
-    "lift_gesummv_allgather": (i32, [i64, i64, f32, vp, f32, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, u64, vp]),
-    "lift_atax_reduce": (i32, [i64, i64, vp, vp, vp, vp, sz, vp, i32, i32, i32, u64, i32, vp]),
+    "lift_dot_allreduce": (i32, [i64, vp, vp, vp, vp, sz, vp, i32, i32, vp]),
+    "lift_gemv_allgather": (i32, [i64, i64, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, vp]),
+    "lift_gesummv_allgather": (i32, [i64, i64, f32, vp, f32, vp, vp, i64, i64, vp, vp, sz, vp, i32, i32, vp]),
+    "lift_atax_reduce": (i32, [i64, i64, vp, vp, vp, vp, sz, vp, i32, i32, i32, i32, vp]),
     "lift_dot_host": (i32, [i64, vp, vp, vp, vp, vp, vp, vp, sz, vp]),
     "lift_gemv_host": (i32, [i64, i64, vp, vp, vp, vp, vp, vp, vp]),
     "lift_gesummv_host": (i32, [i64, i64, f32, vp, f32, vp, vp, vp, vp, vp, vp, vp, vp]),

@@ -626,11 +626,10 @@ __device__ __forceinline__ void grid_barrier(unsigned int *gbar) {
             __threadfence();  // publish this block's partial row
             atomicAdd(gbar, 1u);
         }
-        unsigned int v;
-        do {
-            v = ld_acquire_gpu(gbar);
-            if (v < gridDim.x) __nanosleep(64);
-        } while (v < gridDim.x);
+        // bounded: blocks that are not all resident (a concurrent kernel holding
+        // SMs under a plain launch) trap after the spin limit instead of hanging
+        SpinDeadline dl;
+        while (ld_acquire_gpu(gbar) < gridDim.x) dl.pause("grid barrier: not every block is resident");
     }
     __syncthreads();
 }
@@ -693,6 +692,14 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     if (tid == 0) {  // prologue: fill the ring (and the L2 prefetch window beyond it)
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
         for (int i = 0; i < l2a; ++i) prefetch_stage(nst + i);
+    }
+    // fused (all-)reduce: this call's epoch; the destinations have finished with
+    // the parity buffer this call writes (checked now, while the ring fills; the
+    // main loop's first block barrier orders the later pushes after it)
+    uint64_t ep = 0;
+    if (ex.world > 0) {
+        ep = exch_epoch(ex);
+        if (tid == 0) exch_wait_consumed_all(ex, dst, ep);
     }
 
     constexpr bool XS = QC >= kFusedXsmemQc;  // x in shared memory (after the ring) instead of registers
@@ -870,7 +877,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     const float4 *y4 = reinterpret_cast<const float4 *>(y);
     for (int q = 0; q < ex.world; ++q) {
         if (dst >= 0 && q != dst) continue;
-        float4 *d4 = reinterpret_cast<float4 *>(exch_data(ex.peers[q], ex) + (int64_t)ex.rank * n);
+        float4 *d4 = reinterpret_cast<float4 *>(exch_data(ex.peers[q], ex, ep) + (int64_t)ex.rank * n);
         for (int64_t c = c0 + threadIdx.x; c < c1; c += blockDim.x) d4[c] = y4[c];
     }
     __syncthreads();
@@ -882,13 +889,15 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         if (last_block) {  // every block has pushed (and passed the grid barrier): re-arm, publish
             gbar[0] = 0u;
             gbar[1] = 0u;
-            exch_signal(ex, dst);
+            exch_signal(ex, dst, ep);
+            // a rank that receives nothing is done with this epoch once it has published
+            if (dst >= 0 && ex.rank != dst) exch_ack(ex, ep);
         }
     }
     if (dst >= 0 && ex.rank != dst) return;
-    if (threadIdx.x == 0) exch_wait_all(ex);
+    if (threadIdx.x == 0) exch_wait_all(ex, ep);
     __syncthreads();
-    const float *src = exch_data(ex.peers[ex.rank], ex);
+    const float *src = exch_data(ex.peers[ex.rank], ex, ep);
     for (int64_t c = c0 + threadIdx.x; c < c1; c += blockDim.x) {
         float4 acc = zero4();
         for (int r = 0; r < ex.world; ++r) {
@@ -899,6 +908,16 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
             acc.w = __fadd_rn(acc.w, ld_volatile(p + 3));
         }
         reinterpret_cast<float4 *>(y)[c] = acc;
+    }
+    // the last block to finish reading acks the epoch (its acquire sees every
+    // other block's reads completed before their release-add)
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned int *readers = exch_readers(ex.peers[ex.rank]);
+        if (atom_acq_rel_add(readers, 1u) == gridDim.x - 1) {
+            *readers = 0u;
+            exch_ack(ex, ep);
+        }
     }
 }
 
@@ -1170,6 +1189,29 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
         *grid_out = (int)(K * C);
         return cudaSuccess;
     }
+    // The grid barrier needs every cluster resident: ask for a cooperative launch
+    // together with the cluster shape (the launch then fails instead of running a
+    // grid that cannot be co-resident).  Where the driver refuses the combination
+    // the launch is plain and the barrier's bounded spin is the backstop.
+    static int coop_ok[64];  // per device: 0 unknown, 1 accepted, -1 refused
+    cudaLaunchAttribute attr2[2] = {attr[0], {}};
+    attr2[1].id = cudaLaunchAttributeCooperative;
+    attr2[1].val.cooperative = 1;
+    const int dev = d.device >= 0 && d.device < 64 ? d.device : 0;
+    if (coop_ok[dev] >= 0) {
+        cfg.attrs = attr2;
+        cfg.numAttrs = 2;
+        cudaError_t e2 = cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
+        if (e2 == cudaSuccess) {
+            coop_ok[dev] = 1;
+            return cudaSuccess;
+        }
+        if (coop_ok[dev] == 1) return e2;
+        (void)cudaGetLastError();  // refused: remember, launch plainly
+        coop_ok[dev] = -1;
+        cfg.attrs = attr;
+        cfg.numAttrs = 1;
+    }
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
 }
 
@@ -1201,7 +1243,8 @@ cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *bloc
 
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     cudaFuncAttributes a;
-    cudaError_t e = cudaFuncGetAttributes(&a, k_atax_fused<1, 4>);
+    cudaError_t e = set_spin_limit_here();
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<1, 4>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<1, 2>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<1, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 2>);

@@ -391,27 +391,26 @@ size_t lift_exchange_bytes(int kind, int64_t len, int world) {
     return (b + 255) / 256 * 256;
 }
 
-static int check_group(void *const *peers, int rank, int world, uint64_t epoch) {
-    if (world < 1 || world > lift::kMaxWorld || rank < 0 || rank >= world || epoch == 0) return LIFT_ERR_BAD_SIZE;
+static int check_group(void *const *peers, int rank, int world) {
+    if (world < 1 || world > lift::kMaxWorld || rank < 0 || rank >= world) return LIFT_ERR_BAD_SIZE;
     if (peers == nullptr) return LIFT_ERR_NULL_PTR;
     if ((reinterpret_cast<uintptr_t>(peers) & 7) != 0) return LIFT_ERR_MISALIGNED;
     return LIFT_OK;
 }
 
-static lift::Exch make_exch(void *const *peers, int rank, int world, uint64_t epoch, int64_t cap) {
+static lift::Exch make_exch(void *const *peers, int rank, int world, int64_t cap) {
     lift::Exch e;
     e.peers = reinterpret_cast<char *const *>(peers);
     e.rank = rank;
     e.world = world;
-    e.epoch = epoch;
     e.cap = cap;
     return e;
 }
 
 int lift_dot_allreduce(int64_t n, const float *x, const float *y, float *result, void *workspace,
-                       size_t workspace_bytes, void *const *peers, int rank, int world, uint64_t epoch,
+                       size_t workspace_bytes, void *const *peers, int rank, int world,
                        lift_stream_t stream) {
-    int st = check_group(peers, rank, world, epoch);
+    int st = check_group(peers, rank, world);
     if (st != LIFT_OK) return st;
     if (!size_ok(n, 1)) return LIFT_ERR_BAD_SIZE;
     if (result == nullptr) return LIFT_ERR_NULL_PTR;
@@ -428,14 +427,14 @@ int lift_dot_allreduce(int64_t n, const float *x, const float *y, float *result,
     cudaError_t e = lift::device_info(&d);
     if (e != cudaSuccess) return cuda_status(e);
     return cuda_status(lift::launch_dot(d, n, x, y, result, workspace, (cudaStream_t)stream,
-                                        make_exch(peers, rank, world, epoch, lift::kMaxWorld)));
+                                        make_exch(peers, rank, world, lift::kMaxWorld)));
 }
 
 static int gather_common(int nmat, int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B,
                          const float *x, int64_t row0, int64_t m_total, float *y, void *workspace,
-                         size_t workspace_bytes, void *const *peers, int rank, int world, uint64_t epoch,
+                         size_t workspace_bytes, void *const *peers, int rank, int world,
                          lift_stream_t stream) {
-    int st = check_group(peers, rank, world, epoch);
+    int st = check_group(peers, rank, world);
     if (st != LIFT_OK) return st;
     if (!size_ok(m, n) || !size_ok(m_total, 1) || row0 < 0 || row0 + m > m_total) return LIFT_ERR_BAD_SIZE;
     if (m_total > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
@@ -465,7 +464,7 @@ static int gather_common(int nmat, int64_t m, int64_t n, float alpha, const floa
     g.alpha = alpha;
     g.beta = beta;
     g.epi = nmat == 2 ? lift::kEpiSum2 : lift::kEpiStore;
-    g.ex = make_exch(peers, rank, world, epoch, m_total);
+    g.ex = make_exch(peers, rank, world, m_total);
     g.row0 = row0;
     g.m_total = m_total;
     g.ticket = static_cast<unsigned int *>(workspace);
@@ -474,23 +473,23 @@ static int gather_common(int nmat, int64_t m, int64_t n, float alpha, const floa
 
 int lift_gemv_allgather(int64_t m, int64_t n, const float *A, const float *x, int64_t row0, int64_t m_total,
                         float *y, void *workspace, size_t workspace_bytes, void *const *peers, int rank, int world,
-                        uint64_t epoch, lift_stream_t stream) {
+                        lift_stream_t stream) {
     return gather_common(1, m, n, 1.f, A, 0.f, nullptr, x, row0, m_total, y, workspace, workspace_bytes, peers, rank,
-                         world, epoch, stream);
+                         world, stream);
 }
 
 int lift_gesummv_allgather(int64_t m, int64_t n, float alpha, const float *A, float beta, const float *B,
                            const float *x, int64_t row0, int64_t m_total, float *y, void *workspace,
-                           size_t workspace_bytes, void *const *peers, int rank, int world, uint64_t epoch,
+                           size_t workspace_bytes, void *const *peers, int rank, int world,
                            lift_stream_t stream) {
     return gather_common(2, m, n, alpha, A, beta, B, x, row0, m_total, y, workspace, workspace_bytes, peers, rank,
-                         world, epoch, stream);
+                         world, stream);
 }
 
 int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
-                     size_t workspace_bytes, void *const *peers, int rank, int world, int dst, uint64_t epoch,
+                     size_t workspace_bytes, void *const *peers, int rank, int world, int dst,
                      int blocks, lift_stream_t stream) {
-    int st = check_group(peers, rank, world, epoch);
+    int st = check_group(peers, rank, world);
     if (st != LIFT_OK) return st;
     if (dst < -1 || dst >= world || blocks < 0) return LIFT_ERR_BAD_SIZE;
     if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
@@ -511,7 +510,7 @@ int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float
     cudaError_t e = lift::device_info(&d);
     if (e != cudaSuccess) return cuda_status(e);
     return cuda_status(lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream,
-                                               make_exch(peers, rank, world, epoch, (int64_t)world * n), dst,
+                                               make_exch(peers, rank, world, (int64_t)world * n), dst,
                                                blocks));
 }
 
@@ -608,6 +607,6 @@ const char *lift_strerror(int status) {
 
 const char *lift_last_cuda_error(void) { return g_cuda_err; }
 
-int lift_version(void) { return (1 << 16) | 0; }
+int lift_version(void) { return (2 << 16) | 0; }
 
 }  // extern "C"

@@ -9,10 +9,54 @@
 
 #include <cuda_runtime.h>
 #include <stdint.h>
+#include <stdlib.h>
 
 namespace lift {
 
 constexpr int kWarp = 32;
+
+// ---------------------------------------------------------------------------
+// Bounded spins.  Every in-kernel wait on another block or rank (grid barrier,
+// exchange flags) gives up after a time limit and traps (the launch fails with
+// an error at the caller's next synchronisation) instead of hanging the GPU
+// when its partner can never arrive: blocks that are not co-resident, a peer
+// rank that never makes the matching call.  The limit (default 20 s, far above
+// any legitimate wait: the slowest kernel here takes ~3 ms) comes from
+// LIFT_SPIN_TIMEOUT_MS, read when the library first touches a device.
+// ---------------------------------------------------------------------------
+constexpr unsigned long long kSpinLimitDefaultNs = 20ull * 1000 * 1000 * 1000;
+static __device__ unsigned long long g_spin_limit_ns = kSpinLimitDefaultNs;  // one copy per translation unit
+
+__device__ __forceinline__ unsigned long long globaltimer_ns() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+
+struct SpinDeadline {
+    unsigned long long t0 = 0;
+    // one failed poll: back off; trap once the limit has passed since the first
+    __device__ __forceinline__ void pause(const char * /* what is awaited (documentation) */, unsigned ns = 64) {
+        __nanosleep(ns);
+        const unsigned long long t = globaltimer_ns();
+        if (t0 == 0)
+            t0 = t;
+        else if (t - t0 > g_spin_limit_ns)
+            __trap();
+    }
+};
+
+static inline unsigned long long spin_limit_from_env() {
+    const char *v = getenv("LIFT_SPIN_TIMEOUT_MS");
+    if (v == nullptr || *v == 0) return kSpinLimitDefaultNs;
+    const long long ms = atoll(v);
+    return ms > 0 ? (unsigned long long)ms * 1000000ull : kSpinLimitDefaultNs;
+}
+// sets this translation unit's copy on the current device
+static inline cudaError_t set_spin_limit_here() {
+    const unsigned long long ns = spin_limit_from_env();
+    return cudaMemcpyToSymbol(g_spin_limit_ns, &ns, sizeof ns);
+}
 
 // ---------------------------------------------------------------------------
 // Global loads

@@ -19,10 +19,6 @@
 
 namespace lift {
 
-// ticket hand-off: one atom.acq_rel (true) or __threadfence + atomicAdd (false);
-// tools/fence_probe.py
-constexpr bool kDotAcqRelTicket = true;
-
 template <int TPB, int U>
 __device__ __forceinline__ float block_sum(float v, float *red) {
     constexpr int W = TPB / kWarp;
@@ -100,21 +96,16 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
     if (threadIdx.x == 0) {
         partials[blockIdx.x] = bs;
         // release: publishes this block's partial; acquire: the last block then
-        // sees every other block's (its threads read them after the barrier below)
-        unsigned int t;
-        if constexpr (kDotAcqRelTicket) {
-            t = atom_acq_rel_add(ticket, 1u);
-        } else {
-            __threadfence();
-            t = atomicAdd(ticket, 1u);
-        }
+        // sees every other block's (its threads read them after the barrier below).
+        // One atom.acq_rel instead of __threadfence + atomicAdd (fence.sc is
+        // stronger than needed; tools/fence_probe.py, profiles/r01w_fence_probe.txt)
+        const unsigned int t = atom_acq_rel_add(ticket, 1u);
         am_last = (t == gridDim.x - 1);
     }
     __syncthreads();
     if (!am_last) return;
     // second stage (L422-426), fixed order: thread j folds partials j, j+TPB, ...
     // (8 predicated loads in flight, added in that order)
-    if constexpr (!kDotAcqRelTicket) __threadfence();
     float p = 0.f;
     for (int j0 = threadIdx.x; j0 < (int)gridDim.x; j0 += 8 * TPB) {
         float v[8];
@@ -135,14 +126,17 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
             // fused all-reduce (NEXT-2): this rank's partial into slot `rank` of every
             // rank's exchange area, publish, wait for all ranks, then every rank sums
             // the slots in rank order: bitwise identical results on all ranks
-            for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex)[ex.rank] = tot;
+            const uint64_t ep = exch_epoch(ex);
+            exch_wait_consumed_all(ex, -1, ep);
+            for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex, ep)[ex.rank] = tot;
             __threadfence_system();
-            exch_signal(ex, -1);
-            exch_wait_all(ex);
-            const float *d = exch_data(ex.peers[ex.rank], ex);
+            exch_signal(ex, -1, ep);
+            exch_wait_all(ex, ep);
+            const float *d = exch_data(ex.peers[ex.rank], ex, ep);
             float sum = 0.f;
             for (int r = 0; r < ex.world; ++r) sum = __fadd_rn(sum, ld_volatile(d + r));
             *result = sum;
+            exch_ack(ex, ep);
         }
     }
 }
@@ -192,7 +186,8 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
 // spinning on a peer's flag, as the fused collectives do, would never let it).
 cudaError_t preload_dot() {
     cudaFuncAttributes a;
-    cudaError_t e = cudaFuncGetAttributes(&a, k_dot<kDotTPB, kDotU, true>);
+    cudaError_t e = set_spin_limit_here();
+    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_dot<kDotTPB, kDotU, true>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_dot<kDotTPB, kDotU, false>);
     return e;
 }

@@ -3,32 +3,56 @@
 // NVLink (peer pointers from torch symmetric memory / CUDA IPC), a release
 // flag per (rank, epoch), and acquire-spins on the receiving side.
 //
-// Exchange area of every rank (same layout and size on all ranks):
-//   [0, 512)      uint64 flag[64]   flag[r] = last epoch whose data rank r has
-//                                   finished writing into THIS area
-//   [1024, ...)   float data[2][cap] double-buffered by epoch parity
-// A rank can be at most one epoch ahead of any peer (every call waits for all
-// peers' flags of its own epoch), so parity double-buffering never lets a
-// fast rank overwrite data a slow rank has not consumed yet.
+// Exchange area of every rank (same layout and size on all ranks, zero before
+// the first call):
+//   [0, 512)      uint64 flag[64]  flag[r] = last epoch whose data rank r has
+//                                  finished writing into THIS area
+//   [512, 1024)   uint64 ack[64]   ack[r] = last epoch rank r has finished
+//                                  with (its own reads of that epoch's data
+//                                  from its own area are done); every rank
+//                                  writes its ack into EVERY rank's area
+//   [1024, 1028)  uint32           readers' departure counter (multi-block
+//                                  consumers; zero between calls)
+//   [2048, ...)   float data[2][cap]  double-buffered by epoch parity
+//
+// The epoch lives on the device: a call's epoch is ack[rank] of the caller's
+// own area + 1 (its previous call acked epoch e - 1 there as its last act), so
+// the host passes no counter and a step of fused collectives can be captured
+// in a CUDA graph and replayed.
+//
+// Buffer reuse: the data of epoch e goes to parity e & 1, last used by epoch
+// e - 2.  Before rank p stores epoch e's data into rank q's area it waits
+// until ack[q] (in p's OWN area, written there by q) >= e - 2, i.e. q has
+// finished reading epoch e - 2.  This holds in every mode — all-gather,
+// all-reduce and reduce-to-one-rank, where the senders do not wait for the
+// destination and could otherwise run two calls ahead — and in any mix of
+// them.  The check is a local load, normally satisfied at the first read.
 #pragma once
 
 #include <stdint.h>
 
+#include "common.cuh"
+
 namespace lift {
 
 constexpr int kMaxWorld = 64;
-constexpr size_t kExchHeader = 1024;
+constexpr size_t kExchHeader = 2048;
+constexpr size_t kExchAckOff = 512;
+constexpr size_t kExchReadersOff = 1024;
 
 struct Exch {
     char *const *peers = nullptr;  // device array [world]: each rank's exchange area (this process's mapping)
     int rank = 0, world = 0;       // world == 0: no exchange (plain kernel)
-    unsigned long long epoch = 0;  // >= 1, the same sequence of calls on every rank
     int64_t cap = 0;               // floats per parity buffer
 };
 
 __device__ __forceinline__ uint64_t *exch_flags(char *area) { return reinterpret_cast<uint64_t *>(area); }
-__device__ __forceinline__ float *exch_data(char *area, const Exch &e) {
-    return reinterpret_cast<float *>(area + kExchHeader) + (int64_t)(e.epoch & 1ull) * e.cap;
+__device__ __forceinline__ uint64_t *exch_acks(char *area) { return reinterpret_cast<uint64_t *>(area + kExchAckOff); }
+__device__ __forceinline__ unsigned int *exch_readers(char *area) {
+    return reinterpret_cast<unsigned int *>(area + kExchReadersOff);
+}
+__device__ __forceinline__ float *exch_data(char *area, const Exch &e, uint64_t epoch) {
+    return reinterpret_cast<float *>(area + kExchHeader) + (int64_t)(epoch & 1ull) * e.cap;
 }
 
 __device__ __forceinline__ void st_release_sys(uint64_t *p, uint64_t v) {
@@ -39,31 +63,56 @@ __device__ __forceinline__ uint64_t ld_acquire_sys(const uint64_t *p) {
     asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
     return v;
 }
+__device__ __forceinline__ uint64_t ld_relaxed_sys(const uint64_t *p) {
+    uint64_t v;
+    asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
 __device__ __forceinline__ float ld_volatile(const float *p) {
     float v;
     asm volatile("ld.volatile.global.f32 %0, [%1];" : "=f"(v) : "l"(p) : "memory");
     return v;
 }
 
-// After this rank's data stores to the peers: publish (caller did fence.sys).
-__device__ __forceinline__ void exch_signal(const Exch &e, int dst /* -1: all ranks */) {
-    for (int p = 0; p < e.world; ++p)
-        if (dst < 0 || p == dst) st_release_sys(exch_flags(e.peers[p]) + e.rank, (uint64_t)e.epoch);
+// This call's epoch: one more than the last epoch this rank acked into its own area.
+__device__ __forceinline__ uint64_t exch_epoch(const Exch &e) {
+    return ld_relaxed_sys(exch_acks(e.peers[e.rank]) + e.rank) + 1ull;
 }
 
-// Wait until every rank has published epoch e.epoch into THIS rank's area.
-// Bounded: a peer that never arrives (a programming error) traps after ~1
-// minute instead of hanging the GPU; host-side skew between ranks (allocation,
-// pinning, GC) stays far below that.
-__device__ __forceinline__ void exch_wait_all(const Exch &e) {
+// Before storing epoch `epoch`'s data into rank q's area: q has finished with
+// epoch - 2 (the last user of this parity buffer).  Bounded like every spin.
+__device__ __forceinline__ void exch_wait_consumed(const Exch &e, int q, uint64_t epoch) {
+    const uint64_t *a = exch_acks(e.peers[e.rank]) + q;
+    SpinDeadline dl;
+    while (ld_acquire_sys(a) + 2ull < epoch) dl.pause("exchange: peer never consumed an earlier epoch");
+}
+__device__ __forceinline__ void exch_wait_consumed_all(const Exch &e, int dst /* -1: all ranks */, uint64_t epoch) {
+    for (int q = 0; q < e.world; ++q)
+        if (dst < 0 || q == dst) exch_wait_consumed(e, q, epoch);
+}
+
+// After this rank's data stores to the peers: publish (caller did fence.sys).
+__device__ __forceinline__ void exch_signal(const Exch &e, int dst /* -1: all ranks */, uint64_t epoch) {
+    for (int p = 0; p < e.world; ++p)
+        if (dst < 0 || p == dst) st_release_sys(exch_flags(e.peers[p]) + e.rank, epoch);
+}
+
+// Wait until every rank has published `epoch` into THIS rank's area.  Bounded:
+// a peer that never arrives (a programming error) traps instead of hanging the
+// GPU; host-side skew between ranks (allocation, pinning, GC) stays far below
+// the limit.
+__device__ __forceinline__ void exch_wait_all(const Exch &e, uint64_t epoch) {
     const uint64_t *f = exch_flags(e.peers[e.rank]);
-    const long long t0 = clock64();
-    for (int r = 0; r < e.world; ++r) {
-        while (ld_acquire_sys(f + r) < (uint64_t)e.epoch) {
-            __nanosleep(100);
-            if (clock64() - t0 > (1ll << 37)) __trap();  // ~70 s at 1.96 GHz
-        }
-    }
+    SpinDeadline dl;
+    for (int r = 0; r < e.world; ++r)
+        while (ld_acquire_sys(f + r) < epoch) dl.pause("exchange: a peer never published its data");
+}
+
+// The last act of a call: this rank is done with `epoch` (its reads of its own
+// area are complete).  Written into every rank's area; the own copy is also
+// the next call's epoch base.
+__device__ __forceinline__ void exch_ack(const Exch &e, uint64_t epoch) {
+    for (int p = 0; p < e.world; ++p) st_release_sys(exch_acks(e.peers[p]) + e.rank, epoch);
 }
 
 }  // namespace lift

@@ -86,6 +86,15 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     const int64_t kfull = nv / kVLanes;                   // k-steps whose every vector is in the row
     const int lane_off = kWarp * (wr * KQ) + lane;        // first virtual lane of this lane, slice q adds 32*q
 
+    // fused all-gather: this call's epoch, and every destination has finished
+    // with the parity buffer this call writes (the barrier orders the row
+    // writers after the check)
+    uint64_t ep = 0;
+    if (ex.world > 0) {
+        ep = exch_epoch(ex);
+        if (threadIdx.x == 0) exch_wait_consumed_all(ex, -1, ep);
+        __syncthreads();
+    }
     bool x_pending = false;
     if constexpr (XSMEM) {
         stage_issue(xs, x, (uint32_t)(n * 4), bar);  // toLocal(x), one bulk copy per block
@@ -227,7 +236,7 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
                     if (ex.world == 0) {
                         y[row] = val;
                     } else {  // fused all-gather (NEXT-2): the row goes straight to every rank
-                        for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex)[row0 + row] = val;
+                        for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex, ep)[row0 + row] = val;
                     }
                 }
                 if (nrow >= m) break;
@@ -259,12 +268,14 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
         if (!am_last) return;
         if (threadIdx.x == 0) {
             *ticket = 0u;
-            exch_signal(ex, -1);
-            exch_wait_all(ex);
+            exch_signal(ex, -1, ep);
+            exch_wait_all(ex, ep);
         }
         __syncthreads();
-        const float *src = exch_data(ex.peers[ex.rank], ex);
+        const float *src = exch_data(ex.peers[ex.rank], ex, ep);
         for (int64_t i = threadIdx.x; i < m_total; i += blockDim.x) y[i] = ld_volatile(src + i);
+        __syncthreads();  // every read of this epoch's data is done
+        if (threadIdx.x == 0) exch_ack(ex, ep);
     }
 }
 
@@ -335,7 +346,8 @@ static cudaError_t preload_set() {
 }
 
 cudaError_t preload_gemv() {  // see preload_dot (dot.cu)
-    cudaError_t e = preload_set<1, 4, true, 4>();
+    cudaError_t e = set_spin_limit_here();
+    if (e == cudaSuccess) e = preload_set<1, 4, true, 4>();
     if (e == cudaSuccess) e = preload_set<1, 4, true, 8>();
     if (e == cudaSuccess) e = preload_set<1, 4, false, 4>();
     if (e == cudaSuccess) e = preload_set<1, 4, false, 8>();
@@ -351,8 +363,11 @@ cudaError_t preload_gemv() {  // see preload_dot (dot.cu)
 
 cudaError_t launch_gemv(const DeviceInfo &d, const GemvArgs &a, GemvConfig cfg, cudaStream_t s) {
     const int64_t m = a.m, n = a.n;
-    if (m == 0) return cudaSuccess;
-    if (n == 0) {
+    // with a fused all-gather every rank launches, even with no rows or columns of
+    // its own: its peers wait for its flag (an empty row sums to 0)
+    const bool exch = a.ex.world > 0;
+    if (m == 0 && !exch) return cudaSuccess;
+    if (n == 0 && !exch) {
         if (a.epi == kEpiStore) return cudaMemsetAsync(a.y, 0, (size_t)m * sizeof(float), s);
         // y = 0 + beta*y (and 0 when beta == 0): handled by the kernel with an empty row
     }
@@ -364,7 +379,7 @@ cudaError_t launch_gemv(const DeviceInfo &d, const GemvArgs &a, GemvConfig cfg, 
     // 256-thread block (8 warps x 1 slice each), 4 vector loads per lane per batch, x in
     // SMEM only while >= 4 blocks per SM still fit (a 128 KiB x that pins one block per SM
     // loses ~25 %; L1 serves it better).
-    bool xsmem = vec && 4 * (x_bytes + 1024) <= (size_t)d.smem_per_sm;
+    bool xsmem = vec && m > 0 && 4 * (x_bytes + 1024) <= (size_t)d.smem_per_sm;
     if (cfg.xsmem == 0) xsmem = false;
     if (cfg.xsmem == 1) {
         if (!(vec && x_bytes + 1024 <= (size_t)d.smem_optin)) return cudaErrorInvalidValue;

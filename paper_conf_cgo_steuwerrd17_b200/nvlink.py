@@ -4,8 +4,9 @@ Each rank's kernel writes its results straight into every destination
 rank's exchange area (NVLink peer stores), publishes a flag, and the
 receivers combine contributions in rank order.  An :class:`ExchangeArea`
 holds one rank's view: its own area, the device array of every rank's area
-pointer, and the epoch counter (calls on one area must happen in the same
-order on every rank).
+pointers.  Calls on one area must happen in the same order on every rank; the
+call counter (epoch) lives in the area itself on the device, so a sequence of
+fused calls can be captured in a CUDA graph and replayed.
 
 * :meth:`ExchangeArea.symmetric` — one area per rank from torch symmetric
   memory (multi-GPU, one process per GPU).
@@ -29,7 +30,6 @@ class ExchangeArea:
         self.kind, self.length = kind, length
         self.area, self.peers = area, peers  # keep the allocations alive
         self.rank, self.world = rank, world
-        self.epoch = 0
 
     @staticmethod
     def nbytes(kind: int, length: int, world: int) -> int:
@@ -117,10 +117,6 @@ class ExchangeArea:
         peers = torch.tensor([a.data_ptr() for a in areas], dtype=torch.int64, device=device)
         return [cls(kind, length, areas[r], peers, r, world) for r in range(world)]
 
-    def next_epoch(self) -> int:
-        self.epoch += 1
-        return self.epoch
-
 
 def workspace_bytes(op: str, m: int = 0, n: int = 0) -> int:
     """Workspace bytes of one call (allocate zeroed, reuse across calls)."""
@@ -153,7 +149,7 @@ def lift_dot_allreduce(x: torch.Tensor, y: torch.Tensor, ex: ExchangeArea, out: 
         ws = workspace if workspace is not None else _workspace(f"dotar{ex.rank}", dev,
                                                                 L.lift_dot_workspace_bytes(n), zero=True)
         check(L.lift_dot_allreduce(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
-                                   ex.peers.data_ptr(), ex.rank, ex.world, ex.next_epoch(), _stream(dev)))
+                                   ex.peers.data_ptr(), ex.rank, ex.world, _stream(dev)))
     return out
 
 
@@ -174,13 +170,13 @@ def lift_gemv_allgather(A: torch.Tensor, x: torch.Tensor, row0: int, m_total: in
         ws = workspace if workspace is not None else _workspace(f"gather{ex.rank}", dev, 256, zero=True)
         if B is None:
             st = L.lift_gemv_allgather(m, n, A.data_ptr(), x.data_ptr(), row0, m_total, out.data_ptr(), ws.data_ptr(),
-                                       ws.numel(), ex.peers.data_ptr(), ex.rank, ex.world, ex.next_epoch(),
+                                       ws.numel(), ex.peers.data_ptr(), ex.rank, ex.world,
                                        _stream(dev))
         else:
             _check_tensor(B, "B", 2)
             st = L.lift_gesummv_allgather(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
                                           row0, m_total, out.data_ptr(), ws.data_ptr(), ws.numel(),
-                                          ex.peers.data_ptr(), ex.rank, ex.world, ex.next_epoch(), _stream(dev))
+                                          ex.peers.data_ptr(), ex.rank, ex.world, _stream(dev))
         check(st)
     return out
 
@@ -200,5 +196,5 @@ def lift_atax_reduce(A: torch.Tensor, x: torch.Tensor, ex: ExchangeArea, dst: in
         ws = workspace if workspace is not None else _workspace(f"ataxr{ex.rank}", dev,
                                                                 L.lift_atax_workspace_bytes(m, n), zero=True)
         check(L.lift_atax_reduce(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
-                                 ex.peers.data_ptr(), ex.rank, ex.world, dst, ex.next_epoch(), blocks, _stream(dev)))
+                                 ex.peers.data_ptr(), ex.rank, ex.world, dst, blocks, _stream(dev)))
     return out

@@ -50,7 +50,7 @@ def test_sm100a_cubin_only():
 
 
 def test_version_and_strerror():
-    assert L.lift_version() >> 16 == 1
+    assert L.lift_version() >> 16 == 2
     for s in range(7):
         msg = L.lift_strerror(s).decode()
         assert msg.startswith("LIFT_")
@@ -221,21 +221,21 @@ def test_sgemv_validation():
 def test_nvlink_validation():
     peers = P * 400
     ws = L.lift_dot_workspace_bytes(100)
-    assert L.lift_exchange_bytes(0, 0, 8) >= 1024 + 2 * 64 * 4
+    assert L.lift_exchange_bytes(0, 0, 8) >= 2048 + 2 * 64 * 4
     assert L.lift_exchange_bytes(1, 65536, 8) >= 2 * 65536 * 4
     assert L.lift_exchange_bytes(2, 8192, 8) >= 2 * 8 * 8192 * 4
     assert L.lift_exchange_bytes(3, 10, 8) == 0 and L.lift_exchange_bytes(0, 1, 65) == 0
-    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers, 0, 2, 0, None) == SIZE   # epoch 0
-    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers, 2, 2, 1, None) == SIZE   # rank >= world
-    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, None, 0, 2, 1, None) == NULL
-    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers + 4, 0, 2, 1, None) == MIS
-    assert L.lift_gemv_allgather(10, 4, A_, X_, 95, 100, Y_, W_, 256, peers, 0, 2, 1, None) == SIZE  # rows past m_total
-    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, A_, W_, 256, peers, 0, 2, 1, None) == ALIAS
-    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, Y_, W_, 8, peers, 0, 2, 1, None) == WS
-    assert L.lift_gesummv_allgather(10, 4, 1.0, A_, 1.0, None, X_, 0, 10, Y_, W_, 256, peers, 0, 1, 1, None) == NULL
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers, 0, 0, None) == SIZE      # world 0
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers, 2, 2, None) == SIZE      # rank >= world
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, None, 0, 2, None) == NULL
+    assert L.lift_dot_allreduce(100, X_, Y_, P * 300, W_, ws, peers + 4, 0, 2, None) == MIS
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 95, 100, Y_, W_, 256, peers, 0, 2, None) == SIZE  # rows past m_total
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, A_, W_, 256, peers, 0, 2, None) == ALIAS
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, Y_, W_, 8, peers, 0, 2, None) == WS
+    assert L.lift_gesummv_allgather(10, 4, 1.0, A_, 1.0, None, X_, 0, 10, Y_, W_, 256, peers, 0, 1, None) == NULL
     wsa = L.lift_atax_workspace_bytes(64, 512)
-    assert L.lift_atax_reduce(64, 512, A_, X_, Y_, W_, wsa, peers, 0, 2, 2, 1, 0, None) == SIZE      # dst >= world
-    assert L.lift_atax_reduce(64, 510, A_, X_, Y_, W_, wsa, peers, 0, 2, 0, 1, 0, None) == SIZE     # n % 4
+    assert L.lift_atax_reduce(64, 512, A_, X_, Y_, W_, wsa, peers, 0, 2, 2, 0, None) == SIZE      # dst >= world
+    assert L.lift_atax_reduce(64, 510, A_, X_, Y_, W_, wsa, peers, 0, 2, 0, 0, None) == SIZE     # n % 4
 
 
 def test_host_entry_validation():

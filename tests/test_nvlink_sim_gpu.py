@@ -120,3 +120,76 @@ def test_atax_reduce_rank_with_no_rows(cuda_device):
     for r in range(world):
         ok, margin = oracle.within_tol(outs[r].cpu().numpy(), ref, mag)
         assert ok, margin
+
+
+def _launch_sequence(world, calls, delay_rank=None, delay_cycles=0):
+    """calls[k](r) launches rank r's k-th call on the current stream.  Every rank
+    issues all its calls back to back with NO host synchronisation between them;
+    `delay_rank`'s stream sleeps before each of its calls, so the other ranks run
+    ahead of it as far as the protocol lets them."""
+    streams = [torch.cuda.Stream() for _ in range(world)]
+    torch.cuda.synchronize()
+    for k in range(len(calls)):
+        for r in range(world):
+            with torch.cuda.stream(streams[r]):
+                if r == delay_rank:
+                    torch.cuda._sleep(delay_cycles)
+                calls[k](r)
+    torch.cuda.synchronize()
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_atax_reduce_dst_back_to_back_no_sync(cuda_device, world):
+    """Reduce-to-one-rank calls back to back, the destination delayed before
+    each: the senders never wait for the destination's data, so without the
+    consumed-epoch acknowledgement they would store call k + 2's partials into
+    the parity buffer the destination is still summing for call k (the race of
+    round 1).  Every call's result must match the oracle for ITS x."""
+    K, dst = 5, 0
+    m, n = 1024, 2048
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    xs = [synth.torch_uniform(100 + k, 0, n, device=cuda_device) for k in range(K)]
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
+    parts = [partition_rows(m, world, r) for r in range(world)]
+    ws = [torch.zeros(nvlink.workspace_bytes("atax", m, n), dtype=torch.uint8, device=cuda_device)
+          for _ in range(world)]
+    outs = [[torch.full((n,), float("nan"), device=cuda_device) for _ in range(world)] for _ in range(K)]
+    blocks = 148 // (world + 1)
+    calls = [lambda r, k=k: nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], xs[k], exs[r], dst=dst,
+                                                    blocks=blocks, out=outs[k][r], workspace=ws[r])
+             for k in range(K)]
+    _launch_sequence(world, calls, delay_rank=dst, delay_cycles=400_000)  # ~0.2 ms per call
+    An = A.cpu().numpy()
+    for k in range(K):
+        ref, mag = oracle.atax(An, xs[k].cpu().numpy())
+        ok, margin = oracle.within_tol(outs[k][dst].cpu().numpy(), ref, mag)
+        assert ok, (k, margin)
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_mixed_collectives_back_to_back_no_sync(cuda_device, world):
+    """All-reduce, reduce-to-rank-1 and reduce-to-rank-0 ATAX calls interleaved on
+    one exchange area, back to back, a different rank delayed each time: the
+    device-resident epoch and the acknowledgements keep every call's data apart."""
+    m, n = 600, 1024
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    modes = [-1, 1, 0, 1, -1, 0, 0]
+    K = len(modes)
+    xs = [synth.torch_uniform(200 + k, 0, n, device=cuda_device) for k in range(K)]
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
+    parts = [partition_rows(m, world, r) for r in range(world)]
+    ws = [torch.zeros(nvlink.workspace_bytes("atax", m, n), dtype=torch.uint8, device=cuda_device)
+          for _ in range(world)]
+    outs = [[torch.full((n,), float("nan"), device=cuda_device) for _ in range(world)] for _ in range(K)]
+    blocks = 148 // (world + 1)
+    calls = [lambda r, k=k: nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], xs[k], exs[r], dst=modes[k],
+                                                    blocks=blocks, out=outs[k][r], workspace=ws[r])
+             for k in range(K)]
+    for delayed in range(world):
+        _launch_sequence(world, calls, delay_rank=delayed, delay_cycles=300_000)
+        An = A.cpu().numpy()
+        for k in range(K):
+            ref, mag = oracle.atax(An, xs[k].cpu().numpy())
+            for r in (range(world) if modes[k] < 0 else [modes[k]]):
+                ok, margin = oracle.within_tol(outs[k][r].cpu().numpy(), ref, mag)
+                assert ok, (delayed, k, r, margin)
