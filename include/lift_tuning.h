@@ -19,28 +19,19 @@
  *
  * lift_atax_fused_tuned: lift_atax with the single-pass fused kernel
  * (lift_atax_algo_run(LIFT_ATAX_FUSED, ...): same arguments, workspace and
- * validation; for any nst / l2_ahead the results are bitwise identical to it —
- * the summation order depends only on (m, n), the SM count and the row
- * assignment):
- *   nst       stages (one bulk copy of ~32 KiB of rows each) in the shared-
- *             memory ring, 2..16 and within the shared-memory budget
- *             (0 = automatic)
- *   l2_ahead  stages prefetched into L2 (cp.async.bulk.prefetch) beyond the
- *             ring, 0..64 (-1 = automatic)
+ * validation):
+ *   nst       stages in the shared-memory ring (one bulk copy of ~32 KiB of
+ *             rows each up to 16384 columns, one row slice each for the
+ *             wider, cluster kernel), 2..16 and within the shared-memory
+ *             budget (0 = automatic).  Only the speed changes: results are
+ *             bitwise those of lift_atax_algo_run(LIFT_ATAX_FUSED, ...) for
+ *             every accepted nst, at every width.
  *   cyclic    1 = block b streams row stages b, b+G, b+2G, ... (G blocks),
- *             0 = block b streams one contiguous band of rows (-1 = automatic);
- *             this changes which rows each block's partial sums, so results
- *             are bitwise those of the untuned call only at the automatic
- *             setting
- *   cluster   second stage (the sum of the per-block partial rows of y):
- *             1 = grid barrier of a cooperative launch of one block per SM,
- *             then every block sums a column slice over all partial rows;
- *             2, 4, 8 or 16 = thread-block clusters of that size fold their
- *             partial rows through distributed shared memory into one row
- *             per cluster, and per column slice the last cluster to arrive
- *             sums the cluster rows (the grid is the number of such clusters
- *             that fit at once); 0 = automatic.  Like `cyclic`, this changes
- *             the summation order: bitwise the untuned call only at 0
+ *             0 = block b streams one contiguous band of rows (-1 = automatic,
+ *             which is 1).  This changes which rows each block's partial sums,
+ *             so results are bitwise those of the untuned call only at 1 / -1.
+ *             Rows wider than 16384 (the cluster kernel) are always assigned
+ *             cyclically: 0 is refused there.
  *
  * An unsupported combination returns LIFT_ERR_CUDA with
  * lift_last_cuda_error() = "invalid argument".
@@ -62,15 +53,15 @@ LIFT_API int lift_gesummv_tuned(int64_t m, int64_t n, float alpha, const float *
                        int wpr, int rg, int blocks, int xsmem, int lb, lift_stream_t stream);
 
 LIFT_API int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y,
-                                   void *workspace, size_t workspace_bytes, int nst, int l2_ahead, int cyclic,
-                                   int cluster,
+                                   void *workspace, size_t workspace_bytes, int nst, int cyclic,
                                    lift_stream_t stream);
 
 /* lift_atax_fused_grid: the launch shape of lift_atax's single pass for an
  * m x n matrix on the current device, without launching anything: *blocks
  * thread blocks in clusters of *cluster (1 = no cluster: one block per SM,
- * rows up to 16384 wide; 2..16 = the wide-row kernel, as many clusters as the
- * device's cluster occupancy allows — the GPC layout of the part decides it).
+ * rows up to 16384 wide, a cooperative launch; 2..16 = the wide-row kernel,
+ * as many clusters as the device's cluster occupancy allows — the GPC layout
+ * of the part decides it —, launched cooperative with its cluster shape).
  * LIFT_ERR_BAD_SIZE for shapes the single pass does not take (m < 1, n not a
  * supported width), LIFT_ERR_NULL_PTR for NULL outputs, LIFT_ERR_CUDA when
  * there is no device. */

@@ -207,8 +207,8 @@ def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None,
 
 
 def lift_atax_fused_tuned(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None, nst: int = 0,
-                          l2_ahead: int = -1, cyclic: int = -1, cluster: int = 0) -> torch.Tensor:
-    """lift_atax(algo="fused") with the ring depth / L2 prefetch distance overridden (lift_tuning.h)."""
+                          cyclic: int = -1) -> torch.Tensor:
+    """lift_atax(algo="fused") with the ring depth / row assignment overridden (lift_tuning.h)."""
     _check_tensor(A, "A", 2)
     _check_tensor(x, "x", 1)
     dev = _same_device(A, x)
@@ -223,7 +223,7 @@ def lift_atax_fused_tuned(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | 
     with _on(dev):
         ws = _workspace("atax", dev, nbytes, zero=True)
         check(L.lift_atax_fused_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), ws.data_ptr(), ws.numel(),
-                                      nst, l2_ahead, cyclic, cluster, _stream(dev)))
+                                      nst, cyclic, _stream(dev)))
     return out
 
 

@@ -63,7 +63,7 @@ SIGNATURES = {
     "lift_version": (i32, []),
     "lift_gemv_tuned": (i32, [i64, i64, vp, vp, vp, i32, i32, i32, i32, i32, vp]),
     "lift_gesummv_tuned": (i32, [i64, i64, f32, vp, f32, vp, vp, vp, i32, i32, i32, i32, i32, vp]),
-    "lift_atax_fused_tuned": (i32, [i64, i64, vp, vp, vp, vp, sz, i32, i32, i32, i32, vp]),
+    "lift_atax_fused_tuned": (i32, [i64, i64, vp, vp, vp, vp, sz, i32, i32, vp]),
     "lift_atax_fused_grid": (i32, [i64, i64, vp, vp]),
 }
 

@@ -28,7 +28,7 @@
 // reduces a tile of columns over all partial rows.
 //
 // FUSED, WIDE ROWS (n > 16384, k_atax_fused_wide): the columns split over a
-// thread-block cluster; each block streams its column slice of the cluster's
+// thread-block cluster of 2..16 blocks; each block streams its column slice of the cluster's
 // rows, the warps' slice dots are pushed into every block of the cluster by
 // asynchronous remote stores (st.async + mbarrier complete_tx), and each row's
 // rank-1 update is applied one row later from the ring.  Same second stage.
@@ -196,8 +196,8 @@ static cudaError_t column_pass(const DeviceInfo &d, int64_t m, int64_t n, int64_
     const int64_t cblocks = (nv + TPB - 1) / TPB;
     // one resident wave: column blocks x row splits = SMs x blocks per SM
     int per_sm = 0;
-    cudaError_t e = vec ? cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_atax_cols<4, TPB, 8>, TPB, 0)
-                        : cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_atax_cols<1, TPB, 8>, TPB, 0);
+    cudaError_t e = vec ? occupancy_cached(k_atax_cols<4, TPB, 8>, d.device, TPB, 0, &per_sm)
+                        : occupancy_cached(k_atax_cols<1, TPB, 8>, d.device, TPB, 0, &per_sm);
     if (e != cudaSuccess) return e;
     if (per_sm < 1) per_sm = 1;
     int64_t S = (int64_t)d.sms * per_sm / cblocks;
@@ -271,22 +271,16 @@ constexpr int kFusedSmemBudget = 200 * 1024;
 constexpr int kFusedMaxStages = 16;
 constexpr int64_t kFusedMinN = 256;  // below this, rows are too short to stream efficiently
 
-// Cluster form of the fused kernel's second stage (kernel argument clu):
-// cluster sizes up to kFusedMaxCluster; per-slice arrival tickets live in the
-// workspace header at gbar[kClusterTicket + r] (zero before first use, re-armed
-// by the last arrival).
+// largest thread-block cluster of the wide-row kernel
 constexpr int kFusedMaxCluster = 16;
-constexpr int kClusterTicket = 16;
 
 struct FusedPlan {
     int qc;       // float4 columns per thread (1, 2, 4, 8)
     int cr;       // rows per step
     int nst;      // stages (rows) in the ring
-    int l2a;      // stages prefetched into L2 beyond the ring
     int cyc;      // 1: stages assigned to blocks cyclically, 0: contiguous bands
     size_t hdr;   // barrier + reduction header bytes
     size_t smem;  // dynamic smem bytes
-    int clu;      // second stage: cluster size (0 = grid barrier)
 };
 
 // Stage = CR consecutive rows moved by ONE bulk copy; each consumer step takes
@@ -297,16 +291,8 @@ struct FusedPlan {
 // budget of two steps of a[CR][QC]) and the ring holds ~112 KiB.
 constexpr size_t kFusedStageTarget = 32 * 1024;
 constexpr size_t kFusedRingTarget = 112 * 1024;
-constexpr int kFusedL2Ahead = 0;
 constexpr int kFusedCyclic = 1;
-constexpr int kFusedXsmemQc = 8;
-// Second stage by default: the grid barrier (0).  Clusters of C blocks folding
-// their partial rows through DSMEM (tuning option cluster = C) measured slower
-// at every shape (profiles/r01y_atax_cluster_probe.txt): one block per SM packs
-// into fewer SMs as clusters (C = 4 / 8 / 16: 132 / 120 / 112 blocks, and the
-// ring stream needs every SM), and with C = 2 (148 blocks) the last cluster's
-// sum over 74 cluster rows is one serial chain.
-constexpr int kFusedCluster = 0;  // qc at which x moves from registers to shared memory
+constexpr int kFusedXsmemQc = 8;  // qc at which x moves from registers to shared memory
 
 static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}) {
     if (n <= 0 || n % 4 != 0) return false;
@@ -332,28 +318,21 @@ static bool fused_plan(int64_t n, FusedPlan *p, FusedTuning tune = FusedTuning{}
         nst = tune.nst;
     }
     if (hdr + (size_t)nst * stage + xs_bytes > (size_t)kFusedSmemBudget) return false;
-    if (tune.l2a < -1 || tune.l2a > 64 || tune.cyc < -1 || tune.cyc > 1) return false;
+    if (tune.cyc < -1 || tune.cyc > 1) return false;
     p->qc = qc;
     p->cr = cr;
     p->nst = (int)nst;
-    p->l2a = tune.l2a >= 0 ? tune.l2a : kFusedL2Ahead;
     p->cyc = tune.cyc >= 0 ? tune.cyc : kFusedCyclic;
     p->hdr = hdr;
-    if (tune.clu < 0 || tune.clu > kFusedMaxCluster || (tune.clu & (tune.clu - 1)) != 0) return false;
-    p->clu = tune.clu == 0 ? kFusedCluster : (tune.clu == 1 ? 0 : tune.clu);
-    // the drained ring is reused for the final column-sum tile partials (grid-barrier
-    // form) or for this block's partial row and one float4 per thread (cluster form)
+    // the drained ring is reused for the final column-sum tile partials
     const size_t ring = (size_t)nst * stage, tile = (size_t)kFusedWarps * 32 * 4 * sizeof(float);
-    const size_t crow = (size_t)(n + 31) / 32 * 128 + (size_t)kFusedThreads * 16;
-    size_t tail = ring > tile ? ring : tile;
-    if (p->clu > 0 && crow > tail) tail = crow;
-    p->smem = hdr + tail + xs_bytes;
+    p->smem = hdr + (ring > tile ? ring : tile) + xs_bytes;
     return true;
 }
 
 // ---------------------------------------------------------------------------
 // Wide rows (n > 16384: two rows and x no longer fit one block's ring): the
-// columns are split over a thread-block cluster of C blocks.  Block r of a
+// columns are split over a thread-block cluster of C >= 2 blocks.  Block r of a
 // cluster owns the column slice [r*n/C, (r+1)*n/C) of every row its cluster
 // streams, with x and y of that slice in registers; a row's dot is the
 // fixed-order sum of the C blocks' slice dots.
@@ -370,25 +349,21 @@ struct WidePlan {
 constexpr int kWideLag = 1;
 constexpr int kWideLagBufs = 2 * kWideLag + 2;
 constexpr int kWideQc = 8;
-// Rows wider than this take the wide kernel (clusters of 1 up to 16384: no
-// cluster, x in registers, rows one step late from the ring — 8192x12288 65.7
-// against 72.7 us for the single-block kernel, equal at 16384;
-// profiles/r01zd_atax_wide_c1.txt)
-constexpr int64_t kWideMinN = 8192;
+// Rows wider than this take the wide kernel; up to it the single-block kernel
+// (whose x moves to shared memory above 8192) takes every row, tuned or not.
+constexpr int64_t kWideMinN = 16384;
 
 static size_t wide_sums_bytes(int c) {
     return 8 * kWideLagBufs + 4 * kFusedMaxStages + (size_t)kWideLagBufs * c * kFusedWarps * 4;
 }
 
 static bool wide_plan(int64_t n, WidePlan *p, FusedTuning tune = FusedTuning{}) {
-    FusedPlan narrow;
-    (void)narrow;
     if (n <= kWideMinN || n % 4 != 0) return false;  // below: the single-block kernel
-    if (tune.l2a > 0 || tune.clu > 1 || tune.clu < 0) return false;     // no L2 prefetch / cluster second stage
+    if (tune.cyc == 0 || tune.cyc < -1 || tune.cyc > 1) return false;  // rows always go to clusters cyclically
     // the smallest cluster whose slices fit kWideQc float4 columns per thread: slices
     // of 2049..4096 float4 (32..64 KiB of a row) on as many SMs as possible — clusters
     // of 2 fill all 148 SMs (profiles/r01z_atax_wide_cluster_probe.txt)
-    for (int c = 1; c <= kFusedMaxCluster; c *= 2) {
+    for (int c = 2; c <= kFusedMaxCluster; c *= 2) {
         if (n % (4 * c) != 0) continue;  // every slice a whole number of float4 columns
         const int64_t nvs = n / c / 4;
         if (nvs > kWideQc * (int64_t)kFusedThreads) continue;
@@ -499,59 +474,6 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
 }
 
 
-// y[c] = sum_{k < K} P[k][c] for the vector columns c in [c0, c1), by one
-// block, in a fixed order: each pass covers cw = T/g columns with g row
-// groups (contiguous, in order; 8 loads in flight per thread), then the g
-// group sums of a column are added in group order.  The order depends only
-// on (K, c1 - c0).
-__device__ __forceinline__ void colsum_rows(int K, int64_t nv, const float4 *__restrict__ P4,
-                                           float4 *__restrict__ y4, int64_t c0, int64_t c1,
-                                           float4 *part /* smem [kFusedThreads] */) {
-    const int tid = threadIdx.x;
-    const int64_t w = c1 - c0;
-    if (w <= 0) return;
-    int g = w >= kFusedThreads ? 1 : (int)(kFusedThreads / w);
-    if (g > K) g = K;
-    const int cw = kFusedThreads / g;
-    const int col = tid % cw, grp = tid / cw;
-    const int k0 = grp < g ? K * grp / g : 0, k1 = grp < g ? K * (grp + 1) / g : 0;
-    for (int64_t cb = c0; cb < c1; cb += cw) {
-        const int64_t c = cb + col;
-        float4 acc = zero4();
-        if (c < c1) {
-            for (int k = k0; k < k1; k += 8) {
-                float4 v[8];
-#pragma unroll
-                for (int u = 0; u < 8; ++u)
-                    if (k + u < k1) v[u] = __ldcg(P4 + (int64_t)(k + u) * nv + c);
-#pragma unroll
-                for (int u = 0; u < 8; ++u) {
-                    if (k + u < k1) {
-                        acc.x = __fadd_rn(acc.x, v[u].x);
-                        acc.y = __fadd_rn(acc.y, v[u].y);
-                        acc.z = __fadd_rn(acc.z, v[u].z);
-                        acc.w = __fadd_rn(acc.w, v[u].w);
-                    }
-                }
-            }
-        }
-        part[tid] = acc;
-        __syncthreads();
-        if (tid < cw && c < c1) {
-            float4 s = part[tid];
-            for (int j = 1; j < g; ++j) {
-                const float4 v = part[j * cw + tid];
-                s.x = __fadd_rn(s.x, v.x);
-                s.y = __fadd_rn(s.y, v.y);
-                s.z = __fadd_rn(s.z, v.z);
-                s.w = __fadd_rn(s.w, v.w);
-            }
-            y4[c] = s;
-        }
-        __syncthreads();
-    }
-}
-
 // In-warp sums of CR row partials d[0..CR) (one per lane each), as CR
 // butterflies xor 16, 8, 4, 2, 1 would give them, with the first log2(CR)
 // levels folded: at level xor 16 (CR >= 2) the lower half-warp keeps rows
@@ -648,7 +570,7 @@ template <int QC, int CR>
 __global__ void __launch_bounds__(kFusedThreads, 1)
     k_atax_fused(int64_t m, int64_t n, int nst, int hdr, const float *__restrict__ A, const float *__restrict__ x,
                  float *__restrict__ P, float *__restrict__ y, unsigned int *__restrict__ gbar, Exch ex,
-                 int dst, int l2a, int cyc, bool discard_partials, int clu) {
+                 int dst, int cyc, bool discard_partials) {
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t *full = reinterpret_cast<uint64_t *>(smem);
     float *red = reinterpret_cast<float *>(smem + 8 * kFusedMaxStages);  // [2][CR][16]
@@ -677,22 +599,14 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         mbar_arrive_expect_tx(full + slot, bytes);
         bulk_g2s(stage0 + (size_t)slot * stage_floats, A + stage_row(j) * n, bytes, full + slot);
     };
-    // optional deeper pipeline without smem: stage j is prefetched into L2 when
-    // stage j - l2a enters the ring
-    auto prefetch_stage = [&](int64_t j) {
-        if (j >= nstages) return;
-        bulk_prefetch_l2(A + stage_row(j) * n, (uint32_t)((int64_t)stage_rows(j) * n * 4));
-    };
 
     if (tid == 0) {
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         fence_mbar_init();
     }
     __syncthreads();
-    if (tid == 0) {  // prologue: fill the ring (and the L2 prefetch window beyond it)
+    if (tid == 0)  // prologue: fill the ring
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
-        for (int i = 0; i < l2a; ++i) prefetch_stage(nst + i);
-    }
     // fused (all-)reduce: this call's epoch; the destinations have finished with
     // the parity buffer this call writes (checked now, while the ring fills; the
     // main loop's first block barrier orders the later pushes after it)
@@ -734,10 +648,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     auto step = [&](float4(&cur)[CR][QC], float4(&prev)[CR][QC]) -> bool {
         const int rows = stage_rows(k);
         __syncthreads();  // previous stage: partials published, slot consumed
-        if (tid == 0 && prow > 0 && k - 1 + nst < nstages) {
-            issue_stage(k - 1 + nst, pslot);
-            if (l2a > 0) prefetch_stage(k - 1 + nst + l2a);
-        }
+        if (tid == 0 && prow > 0 && k - 1 + nst < nstages) issue_stage(k - 1 + nst, pslot);
         float *rb = red + buf * CR * kFusedWarps;
         if (rows > 0) {
             mbar_wait_parity(full + slot, phase);
@@ -799,54 +710,6 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     for (;;) {
         if (step(ra, rb2)) break;
         if (step(rb2, ra)) break;
-    }
-    if (clu) {
-        // ---- second stage, cluster form: the C blocks of a cluster fold their
-        // partial y rows through distributed shared memory into ONE row per
-        // cluster (block r owns vector-column slice r), then per slice the last
-        // of the K clusters to publish it sums the K cluster rows.  No grid
-        // barrier, no cooperative launch; the order is fixed by (n, C, K). ----
-        float4 *row4 = reinterpret_cast<float4 *>(stage0);  // the drained ring
-#pragma unroll
-        for (int q = 0; q < QC; ++q) {
-            const int64_t c = tid + (int64_t)kFusedThreads * q;
-            if (c < nv) row4[c] = yr[q];
-        }
-        cluster_sync();  // every block's row is in its smem
-        const uint32_t C = cluster_nctarank(), r = cluster_ctarank();
-        const int K = (int)cluster_count_x();
-        const int64_t cid = cluster_id_x();
-        const int64_t c0 = nv * r / C, c1 = nv * (r + 1) / C;
-        float4 *P4 = reinterpret_cast<float4 *>(P);
-        for (int64_t c = c0 + tid; c < c1; c += kFusedThreads) {
-            float4 v[kFusedMaxCluster];
-            const uint32_t la = smem_u32(row4 + c);
-#pragma unroll
-            for (int b = 0; b < kFusedMaxCluster; ++b)
-                if (b < (int)C) v[b] = ld_dsmem4(dsmem_addr_raw(la, b));
-            float4 acc = v[0];
-#pragma unroll
-            for (int b = 1; b < kFusedMaxCluster; ++b) {
-                if (b < (int)C) {
-                    acc.x = __fadd_rn(acc.x, v[b].x);
-                    acc.y = __fadd_rn(acc.y, v[b].y);
-                    acc.z = __fadd_rn(acc.z, v[b].z);
-                    acc.w = __fadd_rn(acc.w, v[b].w);
-                }
-            }
-            __stcg(P4 + cid * nv + c, acc);
-        }
-        cluster_arrive();  // this block's DSMEM reads are done (waited for before exit)
-        __shared__ int is_last;
-        __syncthreads();   // the slice of this cluster's row is written
-        if (tid == 0) is_last = atom_acq_rel_add(gbar + kClusterTicket + r, 1u) == (unsigned)(K - 1);
-        __syncthreads();
-        if (is_last) {
-            colsum_rows(K, nv, P4, reinterpret_cast<float4 *>(y), c0, c1, row4 + (nv + 7) / 8 * 8);
-            if (tid == 0) gbar[kClusterTicket + r] = 0u;  // every cluster has arrived: re-arm
-        }
-        cluster_wait();  // no block leaves while a peer may still read its smem
-        return;
     }
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
 #pragma unroll
@@ -922,8 +785,13 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 }
 
 template <int QC, int CR>
-static cudaLaunchConfig_t fused_cfg(const FusedPlan &p, int blocks, int clu, bool cooperative, cudaStream_t s,
-                                    cudaLaunchAttribute *attr) {
+static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m, int64_t n, const float *A,
+                             const float *x, float *P, float *y, unsigned int *gbar, int blocks, cudaStream_t s,
+                             const Exch &ex, int dst, bool cooperative) {
+    auto k = k_atax_fused<QC, CR>;
+    cudaError_t e = ensure_smem(k, d.device, p.smem);
+    if (e != cudaSuccess) return e;
+    cudaLaunchAttribute attr[1];
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3((unsigned)blocks);
     cfg.blockDim = dim3(kFusedThreads);
@@ -931,71 +799,13 @@ static cudaLaunchConfig_t fused_cfg(const FusedPlan &p, int blocks, int clu, boo
     cfg.stream = s;
     cfg.attrs = attr;
     cfg.numAttrs = 0;
-    if (clu > 0) {  // cluster form: no grid barrier, no co-residency needed
-        attr[0].id = cudaLaunchAttributeClusterDimension;
-        attr[0].val.clusterDim.x = (unsigned)clu;
-        attr[0].val.clusterDim.y = 1;
-        attr[0].val.clusterDim.z = 1;
-        cfg.numAttrs = 1;
-    } else if (cooperative) {  // the in-kernel grid barrier needs every block resident (one per SM)
+    if (cooperative) {  // the in-kernel grid barrier needs every block resident (one per SM)
         attr[0].id = cudaLaunchAttributeCooperative;
         attr[0].val.cooperative = 1;
         cfg.numAttrs = 1;
     }
-    return cfg;
-}
-
-// Clusters of `clu` blocks (one per SM) that fit at once for this plan, cached
-// per (device, kernel shape, smem, clu); 0 if the cluster shape cannot launch.
-template <int QC, int CR>
-static int fused_max_clusters(const DeviceInfo &d, const FusedPlan &p, int clu) {
-    struct Entry {
-        int dev, nst, clu;
-        size_t smem;
-        int k;
-    };
-    static Entry cache[32];
-    static int used = 0;
-    static std::mutex mu;  // host threads may launch concurrently
-    std::lock_guard<std::mutex> lock(mu);
-    for (int i = 0; i < used; ++i)
-        if (cache[i].dev == d.device && cache[i].nst == p.nst && cache[i].clu == clu && cache[i].smem == p.smem)
-            return cache[i].k;
-    auto k = k_atax_fused<QC, CR>;
-    cudaLaunchAttribute attr[1];
-    cudaLaunchConfig_t cfg = fused_cfg<QC, CR>(p, clu * (d.sms / clu), clu, false, 0, attr);
-    int nc = 0;
-    if (cudaOccupancyMaxActiveClusters(&nc, k, &cfg) != cudaSuccess) {
-        (void)cudaGetLastError();
-        nc = 0;
-    }
-    if (used < 32) cache[used++] = Entry{d.device, p.nst, clu, p.smem, nc};
-    return nc;
-}
-
-template <int QC, int CR>
-static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m, int64_t n, const float *A,
-                             const float *x, float *P, float *y, unsigned int *gbar, int blocks, cudaStream_t s,
-                             const Exch &ex, int dst, bool cooperative, int clu) {
-    auto k = k_atax_fused<QC, CR>;
-    cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
-    if (e != cudaSuccess) return e;
-    if (clu > 0) {
-        if (clu > 8) {
-            e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
-            if (e != cudaSuccess) return e;
-        }
-        int64_t K = fused_max_clusters<QC, CR>(d, p, clu);
-        if (K < 1) return cudaErrorInvalidConfiguration;
-        if (K * clu > kMaxSplits) K = kMaxSplits / clu;
-        const int64_t need = (m + clu - 1) / clu;  // at least one row per cluster
-        if (K > need) K = need < 1 ? 1 : need;
-        blocks = (int)(K * clu);
-    }
-    cudaLaunchAttribute attr[1];
-    cudaLaunchConfig_t cfg = fused_cfg<QC, CR>(p, blocks, clu, cooperative, s, attr);
-    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.l2a, p.cyc,
-                              rows_are_lines(P, n), clu);
+    return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.cyc,
+                              rows_are_lines(P, n));
 }
 
 // Wide-row fused ATAX (see WidePlan).  Cluster kc of K streams rows kc, kc+K,
@@ -1140,8 +950,15 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
                             const float *x, float *P, float *y, unsigned int *gbar, cudaStream_t s,
                             int *grid_out = nullptr /* only report the grid, launch nothing */) {
     auto k = k_atax_fused_wide<kWideQc, C>;
-    cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)p.smem);
-    if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+    cudaError_t e = ensure_smem(k, d.device, p.smem);
+    if (e == cudaSuccess && C > 8) {
+        static bool nonportable[64];  // set once per device
+        const int dev = d.device >= 0 && d.device < 64 ? d.device : 0;
+        if (!nonportable[dev]) {
+            e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+            nonportable[dev] = e == cudaSuccess;
+        }
+    }
     if (e != cudaSuccess) return e;
     cudaLaunchAttribute attr[1];
     attr[0].id = cudaLaunchAttributeClusterDimension;
@@ -1221,8 +1038,7 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
 // clusters fit).  Launches nothing.
 cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *blocks, int *cluster) {
     FusedPlan p;
-    WidePlan w0;
-    if (fused_plan(n, &p) && !wide_plan(n, &w0)) {
+    if (fused_plan(n, &p)) {
         int64_t G = d.sms;
         if (G > kMaxSplits) G = kMaxSplits;
         if (G > m) G = m;
@@ -1234,7 +1050,6 @@ cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *bloc
     WidePlan w;
     if (!wide_plan(n, &w) || m < 1) return cudaErrorInvalidValue;
     *cluster = w.clu;
-    if (w.clu == 1) return run_wide<1>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     if (w.clu == 2) return run_wide<2>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     if (w.clu == 4) return run_wide<4>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     if (w.clu == 8) return run_wide<8>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
@@ -1251,43 +1066,31 @@ cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<2, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<4, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused<8, 1>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 1>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 2>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 4>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 8>);
     if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<kWideQc, 16>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 4>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 8>);
-    if (e == cudaSuccess) e = cudaFuncGetAttributes(&a, k_atax_fused_wide<4, 16>);
     return e;
 }
 
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x, float *y,
                               void *ws, cudaStream_t s, Exch ex, int dst, int blocks, FusedTuning tune) {
     if (n == 0) return cudaSuccess;
-    FusedPlan p;
-    // wide rows: the cluster kernel (single rank, default tuning, grid from the
-    // cluster occupancy); explicit tuning and the fused exchanges keep the
-    // single-block kernel where it exists
-    const bool tuned = tune.nst != 0 || tune.l2a > 0 || tune.cyc >= 0 || tune.clu > 1;
-    FusedPlan pdef;
-    const bool narrow_exists = fused_plan(n, &pdef);  // a single-block kernel for this width
+    unsigned int *gbar = static_cast<unsigned int *>(ws);
+    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
+    // rows wider than 16384: the cluster kernel (single rank, grid from the cluster occupancy)
     WidePlan w;
-    if (ex.world == 0 && blocks <= 0 && (!narrow_exists || !tuned) && wide_plan(n, &w, tune)) {
+    if (ex.world == 0 && blocks <= 0 && wide_plan(n, &w, tune)) {
         if (m == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
-        unsigned int *gbar = static_cast<unsigned int *>(ws);
-        float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
-        if (w.clu == 1) return run_wide<1>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 2) return run_wide<2>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 4) return run_wide<4>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 8) return run_wide<8>(d, w, m, n, A, x, P, y, gbar, s);
         if (w.clu == 16) return run_wide<16>(d, w, m, n, A, x, P, y, gbar, s);
         return cudaErrorInvalidValue;
     }
+    FusedPlan p;
     if (!fused_plan(n, &p, tune)) return cudaErrorInvalidValue;
     if (m == 0 && ex.world == 0) return cudaMemsetAsync(y, 0, (size_t)n * 4, s);
-    unsigned int *gbar = static_cast<unsigned int *>(ws);
-    float *P = reinterpret_cast<float *>(static_cast<char *>(ws) + kWsHeader);
     int64_t G = d.sms;
     if (G > kMaxSplits) G = kMaxSplits;
     if (G > m) G = m;
@@ -1296,13 +1099,9 @@ cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const f
     // block count (tests running several ranks on one GPU) launches plainly
     const bool cooperative = blocks <= 0;
     if (blocks > 0) G = blocks < G ? blocks : G;
-    // second stage: clusters of p.clu blocks (single rank, grid chosen from the
-    // cluster occupancy), else the grid barrier (exchanges, explicit grids)
-    const int clu = (ex.world == 0 && blocks <= 0 && m > 0) ? p.clu : 0;
     cudaError_t e = cudaErrorInvalidValue;
-#define LIFT_FUSED_CASE(QC, CR)                                                                                     \
-    if (p.qc == QC && p.cr == CR)                                                                                   \
-        e = run_fused<QC, CR>(d, p, m, n, A, x, P, y, gbar, (int)G, s, ex, dst, cooperative, clu);
+#define LIFT_FUSED_CASE(QC, CR) \
+    if (p.qc == QC && p.cr == CR) e = run_fused<QC, CR>(d, p, m, n, A, x, P, y, gbar, (int)G, s, ex, dst, cooperative);
     // fused_plan pairs: qc 1 -> cr 4 (rows <= 8 KiB), qc 2 -> cr 2, qc 4 / 8 -> cr 1
     LIFT_FUSED_CASE(1, 4)
     LIFT_FUSED_CASE(1, 2)

@@ -241,8 +241,7 @@ int lift_atax_fused_grid(int64_t m, int64_t n, int *blocks, int *cluster) {
 }
 
 int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, float *y, void *workspace,
-                          size_t workspace_bytes, int nst, int l2_ahead, int cyclic, int cluster,
-                          lift_stream_t stream) {
+                          size_t workspace_bytes, int nst, int cyclic, lift_stream_t stream) {
     // validation of lift_atax_algo_run(LIFT_ATAX_FUSED, ...), then the overrides
     if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
     if (n > 0 && y == nullptr) return LIFT_ERR_NULL_PTR;
@@ -266,9 +265,7 @@ int lift_atax_fused_tuned(int64_t m, int64_t n, const float *A, const float *x, 
     if (e != cudaSuccess) return cuda_status(e);
     lift::FusedTuning t;
     t.nst = nst;
-    t.l2a = l2_ahead;
     t.cyc = cyclic;
-    t.clu = cluster;
     return cuda_status(
         lift::launch_atax_fused(d, m, n, A, x, y, workspace, (cudaStream_t)stream, lift::Exch{}, -1, 0, t));
 }

@@ -11,6 +11,8 @@
 #include <stdint.h>
 #include <stdlib.h>
 
+#include <mutex>
+
 namespace lift {
 
 constexpr int kWarp = 32;
@@ -56,6 +58,63 @@ static inline unsigned long long spin_limit_from_env() {
 static inline cudaError_t set_spin_limit_here() {
     const unsigned long long ns = spin_limit_from_env();
     return cudaMemcpyToSymbol(g_spin_limit_ns, &ns, sizeof ns);
+}
+
+// ---------------------------------------------------------------------------
+// Host-side launch helpers, cached per (kernel, device, shape): the CUDA
+// queries cost ~1-3 us of host time each, more than a small launch itself.
+// ---------------------------------------------------------------------------
+struct KernelCache {
+    struct Entry {
+        const void *kern;
+        int dev, threads;
+        size_t smem;
+        int value;
+    };
+    Entry e[256];
+    int used = 0;
+    std::mutex mu;
+};
+static inline KernelCache &kernel_cache() {
+    static KernelCache c;  // one per translation unit is enough (keys include the kernel)
+    return c;
+}
+// cudaOccupancyMaxActiveBlocksPerMultiprocessor, cached
+template <typename K>
+static inline cudaError_t occupancy_cached(K kern, int dev, int threads, size_t smem, int *per_sm) {
+    KernelCache &c = kernel_cache();
+    const void *kp = reinterpret_cast<const void *>(kern);
+    {
+        std::lock_guard<std::mutex> lock(c.mu);
+        for (int i = 0; i < c.used; ++i)
+            if (c.e[i].kern == kp && c.e[i].dev == dev && c.e[i].threads == threads && c.e[i].smem == smem) {
+                *per_sm = c.e[i].value;
+                return cudaSuccess;
+            }
+    }
+    cudaError_t err = cudaOccupancyMaxActiveBlocksPerMultiprocessor(per_sm, kern, threads, smem);
+    if (err != cudaSuccess) return err;
+    std::lock_guard<std::mutex> lock(c.mu);
+    if (c.used < 256) c.e[c.used++] = KernelCache::Entry{kp, dev, threads, smem, *per_sm};
+    return cudaSuccess;
+}
+// cudaFuncAttributeMaxDynamicSharedMemorySize >= smem, set once per (kernel, device)
+template <typename K>
+static inline cudaError_t ensure_smem(K kern, int dev, size_t smem) {
+    if (smem <= 48 * 1024) return cudaSuccess;
+    KernelCache &c = kernel_cache();
+    const void *kp = reinterpret_cast<const void *>(kern);
+    std::lock_guard<std::mutex> lock(c.mu);
+    for (int i = 0; i < c.used; ++i)
+        if (c.e[i].kern == kp && c.e[i].dev == dev && c.e[i].threads == -1) {
+            if (c.e[i].smem >= smem) return cudaSuccess;
+            cudaError_t err = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+            if (err == cudaSuccess) c.e[i].smem = smem;
+            return err;
+        }
+    cudaError_t err = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    if (err == cudaSuccess && c.used < 256) c.e[c.used++] = KernelCache::Entry{kp, dev, -1, smem, 0};
+    return err;
 }
 
 // ---------------------------------------------------------------------------

@@ -163,8 +163,8 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     const int64_t units = vec ? (n >> 2) : n;
     // enough blocks to give every thread its units; at most kWaves resident waves
     int per_sm = 0;
-    cudaError_t e = vec ? cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dot<TPB, U, true>, TPB, 0)
-                        : cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dot<TPB, U, false>, TPB, 0);
+    cudaError_t e = vec ? occupancy_cached(k_dot<TPB, U, true>, d.device, TPB, 0, &per_sm)
+                        : occupancy_cached(k_dot<TPB, U, false>, d.device, TPB, 0, &per_sm);
     if (e != cudaSuccess) return e;
     if (per_sm < 1) per_sm = 1;
     // small n: two units per thread (both loads in flight in the unrolled tail) and

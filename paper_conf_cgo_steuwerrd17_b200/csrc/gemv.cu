@@ -288,12 +288,10 @@ static cudaError_t run_gemv(const DeviceInfo &d, const GemvArgs &a, int blocks, 
     auto kern = k_gemv<NMAT, VEC, WPR, RG, XSMEM, LB>;
     constexpr int threads = RG * WPR * kWarp;
     size_t smem = gemv_x_offset<NMAT, RG>() + (XSMEM ? (size_t)a.n * 4 : 0);
-    if (smem > 48 * 1024) {
-        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        if (e != cudaSuccess) return e;
-    }
+    cudaError_t e = ensure_smem(kern, d.device, smem);
+    if (e != cudaSuccess) return e;
     int per_sm = 0;
-    cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, threads, smem);
+    e = occupancy_cached(kern, d.device, threads, smem, &per_sm);
     if (e != cudaSuccess) return e;
     if (per_sm < 1) return cudaErrorInvalidConfiguration;
     const int64_t groups = (a.m + RG - 1) / RG;

@@ -77,10 +77,10 @@ cudaError_t launch_atax_twopass(const DeviceInfo &d, int64_t m, int64_t n, const
 size_t gemv_t_ws_bytes(int64_t m, int64_t n);
 cudaError_t launch_gemv_t(const DeviceInfo &d, int64_t m, int64_t n, int64_t lda, float alpha, const float *A,
                           const float *x, float beta, float *y, void *ws, cudaStream_t s);
-// FusedTuning: nst = ring stages (0 = planned), l2a = stages prefetched into L2
-// beyond the ring, cyc = 1 cyclic / 0 banded row assignment (-1 = planned)
+// FusedTuning: nst = ring stages (0 = planned), cyc = 1 cyclic / 0 banded row
+// assignment (-1 = planned; the wide-row kernel is always cyclic)
 struct FusedTuning {
-    int nst = 0, l2a = -1, cyc = -1, clu = 0;  // clu: 0 planned, 1 grid barrier, 2..16 cluster size
+    int nst = 0, cyc = -1;
 };
 cudaError_t launch_atax_fused(const DeviceInfo &d, int64_t m, int64_t n, const float *A, const float *x,
                               float *y, void *ws, cudaStream_t s, Exch ex = Exch{}, int dst = -1, int blocks = 0,

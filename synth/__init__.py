@@ -79,6 +79,22 @@ def numpy_uniform(seed: int, start: int, count: int, dist: str = "sym") -> np.nd
     return v.astype(np.float32)  # exact: at most 24 significant bits
 
 
+_WIDE_SALT = 0x5BD1E995
+
+
+def numpy_wide(seed: int, start: int, count: int, emin: int = -140, emax: int = 20) -> np.ndarray:
+    """Wide-dynamic-range fp32 for flat indices [start, start+count): full 24-bit
+    significands, binary exponents uniform in [emin, emax] (the default reaches
+    into the subnormal range below 2^-126) and random signs.  Host side only;
+    for the property tests (no value of the method's arithmetic is involved)."""
+    mant = (numpy_bits(seed, start, count) >> np.uint32(1)).astype(np.float64)  # 23 fraction bits
+    eb = numpy_bits(seed ^ _WIDE_SALT, start, count).astype(np.int64)  # exponent + sign bits
+    e = emin + (eb >> 1) % (emax - emin + 1)
+    sign = np.where(eb & 1, -1.0, 1.0)
+    v = sign * (1.0 + mant * 2.0 ** -23) * np.exp2(e.astype(np.float64))
+    return v.astype(np.float32)  # rounds the subnormal ones (deterministically)
+
+
 def numpy_matrix_rows(seed: int, n_cols: int, r0: int, r1: int, dist: str = "sym") -> np.ndarray:
     """Rows [r0, r1) of the row-major matrix with ``n_cols`` columns."""
     return numpy_uniform(seed, r0 * n_cols, (r1 - r0) * n_cols, dist).reshape(r1 - r0, n_cols)

@@ -111,12 +111,12 @@ def test_tuned_validation():
     assert L.lift_gemv_tuned(-1, 4, A_, X_, Y_, 8, 1, 0, -1, 4, None) == SIZE
     assert L.lift_gesummv_tuned(4, 4, 1.0, A_, 1.0, B_, X_, A_, 8, 1, 0, -1, 4, None) == ALIAS
     ws = L.lift_atax_workspace_bytes(64, 512)
-    assert L.lift_atax_fused_tuned(-1, 512, A_, X_, Y_, W_, ws, 0, -1, -1, 0, None) == SIZE
-    assert L.lift_atax_fused_tuned(64, 512, A_, X_, None, W_, ws, 0, -1, -1, 0, None) == NULL
-    assert L.lift_atax_fused_tuned(64, 512, A_, X_, Y_, W_, ws - 16, 0, -1, -1, 0, None) == WS
-    assert L.lift_atax_fused_tuned(64, 512, A_, X_ + 4, Y_, W_, ws, 0, -1, -1, 0, None) == SIZE  # fused needs 16-B
-    assert L.lift_atax_fused_tuned(64, 510, A_, X_, Y_, W_, ws, 0, -1, -1, 0, None) == SIZE  # and n % 4 == 0
-    assert L.lift_atax_fused_tuned(64, 512, A_, X_, A_, W_, ws, 0, -1, -1, 0, None) == ALIAS
+    assert L.lift_atax_fused_tuned(-1, 512, A_, X_, Y_, W_, ws, 0, -1, None) == SIZE
+    assert L.lift_atax_fused_tuned(64, 512, A_, X_, None, W_, ws, 0, -1, None) == NULL
+    assert L.lift_atax_fused_tuned(64, 512, A_, X_, Y_, W_, ws - 16, 0, -1, None) == WS
+    assert L.lift_atax_fused_tuned(64, 512, A_, X_ + 4, Y_, W_, ws, 0, -1, None) == SIZE  # fused needs 16-B
+    assert L.lift_atax_fused_tuned(64, 510, A_, X_, Y_, W_, ws, 0, -1, None) == SIZE  # and n % 4 == 0
+    assert L.lift_atax_fused_tuned(64, 512, A_, X_, A_, W_, ws, 0, -1, None) == ALIAS
 
 
 def test_atax_fused_grid_validation():

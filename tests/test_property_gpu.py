@@ -17,7 +17,7 @@ SETTINGS = settings(max_examples=30, deadline=None, suppress_health_check=list(H
 shapes = st.tuples(st.integers(0, 300), st.integers(0, 3000))
 offsets = st.integers(0, 3)
 seeds = st.integers(0, 10_000)
-dists = st.sampled_from(["sym", "pos"])
+dists = st.sampled_from(["sym", "pos", "wide"])
 scalars = st.sampled_from([0.0, 1.0, -1.0, 0.5, 1.5, 1.2, -3.25, 1e-3])
 
 
@@ -31,7 +31,12 @@ def dev(a, off=0):
 
 
 def gen(seed, shape, dist):
+    """"sym" U[-1,1), "pos" U[0,1) (both on a 2^-23 / 2^-24 grid), or "wide": full
+    24-bit significands over binary exponents -140..20 (subnormals included),
+    random signs — rounding behaviour the grid inputs never exercise."""
     cnt = int(np.prod(shape)) if len(shape) else 1
+    if dist == "wide":
+        return synth.numpy_wide(seed, 0, cnt).reshape(shape)
     return synth.numpy_uniform(seed, 0, cnt, dist).reshape(shape)
 
 
@@ -58,21 +63,21 @@ def test_gemv_property(cuda_device, mn, off, seed, dist):
 
 
 @SETTINGS
-@given(mn=shapes, off=offsets, seed=seeds, al=scalars, be=scalars)
-def test_gesummv_property(cuda_device, mn, off, seed, al, be):
+@given(mn=shapes, off=offsets, seed=seeds, al=scalars, be=scalars, dist=dists)
+def test_gesummv_property(cuda_device, mn, off, seed, al, be, dist):
     m, n = mn
-    A, B, x = gen(seed, (m, n), "sym"), gen(seed + 1, (m, n), "sym"), gen(seed + 2, (n,), "sym")
+    A, B, x = gen(seed, (m, n), dist), gen(seed + 1, (m, n), dist), gen(seed + 2, (n,), dist)
     got = lift.lift_gesummv(al, dev(A, off), be, dev(B, off), dev(x, off)).cpu().numpy()
     ok(got, *oracle.gesummv(al, A, be, B, x))
 
 
 @SETTINGS
-@given(mn=shapes, off=offsets, seed=seeds, algo=st.sampled_from(["auto", "twopass", "fused"]))
-def test_atax_property(cuda_device, mn, off, seed, algo):
+@given(mn=shapes, off=offsets, seed=seeds, algo=st.sampled_from(["auto", "twopass", "fused"]), dist=dists)
+def test_atax_property(cuda_device, mn, off, seed, algo, dist):
     m, n = mn
     if algo == "fused" and (off != 0 or n % 4 or n > 16384 or m == 0 or n == 0):
         algo = "auto"
-    A, x = gen(seed, (m, n), "sym"), gen(seed + 1, (n,), "sym")
+    A, x = gen(seed, (m, n), dist), gen(seed + 1, (n,), dist)
     got = lift.lift_atax(dev(A, off), dev(x, off), algo=algo).cpu().numpy()
     ok(got, *oracle.atax(A, x))
 

@@ -44,3 +44,17 @@ def test_hadamard_orthogonal():
     H = synth.hadamard(32).astype(np.int64)
     assert np.array_equal(H.T @ H, 32 * np.eye(32, dtype=np.int64))
     assert np.all(H[0] == 1) and np.all(H[:, 0] == 1)
+
+
+def test_numpy_wide_range_and_determinism():
+    v = synth.numpy_wide(3, 0, 200_000)
+    assert v.dtype == np.float32 and np.all(np.isfinite(v))
+    assert np.array_equal(v, synth.numpy_wide(3, 0, 200_000))
+    assert np.array_equal(v[1000:2000], synth.numpy_wide(3, 1000, 1000))  # counter-based: any slice
+    a = np.abs(v[v != 0])
+    assert a.max() < 2.0 ** 21 and a.max() > 2.0 ** 19
+    assert np.mean(a < 2.0 ** -126) > 0.05  # subnormals present
+    assert 0.45 < np.mean(v < 0) < 0.55
+    # full significands: most values are not on the 2^-23-relative grid of U[-1,1)
+    m = np.frexp(a[a >= 2.0 ** -126].astype(np.float64))[0]
+    assert np.mean((m * 2 ** 24) % 2 != 0) > 0.4

@@ -41,9 +41,6 @@ for m, n in ((40, 32), (200, 4096), (300, 8192)):
     A = synth.numpy_matrix_rows(2, n, 0, m)
     x = synth.numpy_uniform(0, 0, n)
     chk(f"atax-fused{m}x{n}", lift.lift_atax(t(A), t(x), algo="fused").cpu().numpy(), *oracle.atax(A, x))
-    for clu in (2, 8):  # thread-block-cluster second stage (DSMEM fold, per-slice tickets)
-        chk(f"atax-fused-cluster{clu}-{m}x{n}", lift.lift_atax_fused_tuned(t(A), t(x), cluster=clu).cpu().numpy(),
-            *oracle.atax(A, x))
 # wide rows: the thread-block-cluster single pass.  600 rows make every cluster refill its ring slots,
 # which the last warp done with a slot does after an atom.acq_rel.cta hand-off on a shared counter:
 # racecheck does not model that hand-off (it flags every refill against the earlier reads of the slot,
