@@ -524,10 +524,11 @@ def run_ours(args) -> None:
             dist.barrier(device_ids=[local_rank]) if args.test_backend == "nccl" else dist.barrier()
         torch.cuda.synchronize()
 
-    # 1 GPU: the K timed steps are one CUDA graph (no host launch gaps between the
-    # kernels); timing events are event-record nodes inside it.  N > 1: eager
-    # launches (NCCL collectives are not captured).
-    use_graph = (not distributed) and not args.eager
+    # The K timed steps are one CUDA graph (no host launch gaps between the kernels;
+    # timing events are event-record nodes inside it): at N = 1, and at N > 1 with the
+    # collectives fused into the kernels (their call counter lives on the device, so
+    # replays stay in step across ranks).  N > 1 over NCCL: eager launches.
+    use_graph = (not distributed or fused) and not args.eager
     run_stream = torch.cuda.Stream(device=dev) if use_graph else torch.cuda.current_stream(dev)
     with torch.cuda.stream(run_stream):
         for _ in range(args.warmup):  # untimed; also creates this stream's workspaces
@@ -750,7 +751,9 @@ def run_ours(args) -> None:
                        "l2": "inputs larger than L2: each step streams ~25 GiB; every operand is evicted by the "
                              "following ops before reuse (no flush kernel in the timed region)",
                        "atax_algo": atax_algo, "alpha": ALPHA, "beta": BETA,
-                       "launch": "cuda-graph of the K timed steps" if use_graph else "eager",
+                       "launch": ("cuda-graph of the K timed steps" +
+                                  (", collectives fused into the kernels" if distributed else "")) if use_graph
+                                 else "eager",
                        "frac_of_peak_per_gpu": round(value / world / peak, 4)},
             "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": gpu_launches,
             "clocks": sampler.summary(), "ops": ops, "table1": table1,

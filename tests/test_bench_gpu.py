@@ -52,5 +52,7 @@ def test_bench_two_ranks_one_device(cuda_device, collectives):
     d = _last_json(r.stdout)
     want = "fused (self-checked against nccl)" if collectives == "auto" else collectives
     assert d["n_gpus"] == 2 and d["config"]["collectives"] == want and d["value"] > 0
+    # fused collectives keep their epoch on the device: the timed steps are one CUDA graph as at N = 1
+    assert d["config"]["launch"].startswith("cuda-graph" if collectives != "nccl" else "eager"), d["config"]["launch"]
     for name, o in d["ops"].items():  # compute-only vs the collective, per op
         assert o["compute_ms"] > 0 and o["collective_ms"] >= 0 and o["compute_GB_s_per_rank"] > 0, name
