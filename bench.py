@@ -256,7 +256,49 @@ def cpu_baseline(min_seconds: float = 10.0) -> dict:
         ts.append(time.perf_counter() - t1)
     return {"value": round(gbs, 3), "unit": "GB/s", "cores": th, "kind": "oracle",
             "sample": desc + f"; {passes} passes in {el:.1f} s",
-            "configs0_dot_2^20_ms": round(1e3 * sorted(ts)[2], 3), "host": host_info()}
+            "configs0_dot_2^20_ms": round(1e3 * sorted(ts)[2], 3), "host": host_info(),
+            "per_config_ms": oracle_per_config()}
+
+
+def oracle_per_config() -> dict:
+    """SURVEY.md 8(d) oracle timing: BASELINE.json configs[0..3] (M1-M4) at their
+    full sizes, the oracle as written on one thread and on all host cores (OpenMP
+    over rows; ATAX's pass 2 over column ranges; the dot over 256 fixed chunks
+    combined in order), median of 5 after one untimed run."""
+    import oracle
+    import synth
+
+    th = oracle.default_threads()
+
+    def med5(f):
+        f()
+        ts = []
+        for _ in range(5):
+            t0 = time.perf_counter()
+            f()
+            ts.append(time.perf_counter() - t0)
+        return round(1e3 * sorted(ts)[2], 3)
+
+    out = {}
+    x, y = synth.numpy_uniform(synth.SEED_X, 0, 1 << 20), synth.numpy_uniform(synth.SEED_Y, 0, 1 << 20)
+    out["M1 dot 2^20 (configs[0])"] = {"single_thread_ms": med5(lambda: oracle.dot(x, y)),
+                                       "all_cores_ms": med5(lambda: oracle.dot_chunked(x, y, 256, th))}
+    A = synth.numpy_matrix_rows(synth.SEED_A, 4096, 0, 4096)
+    xv = synth.numpy_uniform(synth.SEED_X, 0, 4096)
+    out["M2 gemv 4096x4096 (configs[1])"] = {"single_thread_ms": med5(lambda: oracle.gemv(A, xv, threads=1)),
+                                             "all_cores_ms": med5(lambda: oracle.gemv(A, xv, threads=th))}
+    A = synth.numpy_matrix_rows(synth.SEED_A, 8192, 0, 8192)
+    B = synth.numpy_matrix_rows(synth.SEED_B, 8192, 0, 8192)
+    xv = synth.numpy_uniform(synth.SEED_X, 0, 8192)
+    out["M3 gesummv 8192x8192 (configs[2])"] = {
+        "single_thread_ms": med5(lambda: oracle.gesummv(ALPHA, A, BETA, B, xv, threads=1)),
+        "all_cores_ms": med5(lambda: oracle.gesummv(ALPHA, A, BETA, B, xv, threads=th))}
+    del B
+    out["M4 atax 8192x8192 (configs[3])"] = {"single_thread_ms": med5(lambda: oracle.atax(A, xv, threads=1)),
+                                             "all_cores_ms": med5(lambda: oracle.atax(A, xv, threads=th))}
+    return {"threads": th, "method": "median of 5 after one untimed run, full config sizes; single thread = the "
+                                     "oracle as written; all cores = OpenMP over rows (ATAX pass 2: column ranges; "
+                                     "dot: 256 fixed chunks folded in order)", "configs": out}
 
 
 def host_info() -> dict:

@@ -50,6 +50,8 @@ def _load():
         i64 = ctypes.c_int64
         lib.oracle_dot.restype = ctypes.c_double
         lib.oracle_dot.argtypes = [i64, f32p, f32p, f64p]
+        lib.oracle_dot_chunked.restype = ctypes.c_double
+        lib.oracle_dot_chunked.argtypes = [i64, f32p, f32p, f64p, ctypes.c_int, ctypes.c_int]
         lib.oracle_gemv.restype = None
         lib.oracle_gemv.argtypes = [i64, i64, f32p, f32p, f64p, f64p, ctypes.c_int]
         lib.oracle_gesummv.restype = None
@@ -97,6 +99,17 @@ def dot(x, y):
     assert x.shape == y.shape
     mag = ctypes.c_double(0.0)
     s = _load().oracle_dot(x.size, _p32(x), _p32(y), ctypes.byref(mag))
+    return float(s), float(mag.value)
+
+
+def dot_chunked(x, y, chunks: int = 256, threads: int | None = None):
+    """(s, mag): the dot over all host cores — fixed chunks folded in order, the
+    same bits for every thread count (oracle.h, reading R23)."""
+    x, y = _f32(x).ravel(), _f32(y).ravel()
+    assert x.shape == y.shape
+    mag = ctypes.c_double(0.0)
+    s = _load().oracle_dot_chunked(x.size, _p32(x), _p32(y), ctypes.byref(mag), int(chunks),
+                                   threads or default_threads())
     return float(s), float(mag.value)
 
 

@@ -34,6 +34,15 @@ extern "C" {
 /* dot(x, y) = reduce(+, 0, map(x, zip(x, y)))   — L285, Sec. 3.1 */
 double oracle_dot(int64_t n, const float *x, const float *y, double *mag);
 
+/* dot over all host cores (SURVEY.md 8(d) oracle timing variant (ii); reading
+   R23): x*y cut into `chunks` fixed contiguous chunks (chunk k = elements
+   [k*n/chunks, (k+1)*n/chunks)), each an in-order fp64 left fold, the chunk
+   sums then folded in chunk order.  The grouping depends only on (n, chunks),
+   never on `threads`, so every thread count gives the same bits; it differs
+   from oracle_dot only in fp64 association (<= n * 2^-53 * mag). */
+double oracle_dot_chunked(int64_t n, const float *x, const float *y, double *mag,
+                          int chunks, int threads);
+
 /* GEMV y = A x, A m x n row-major (lda = n)    — Table 1 L1030 (CLBlast GEMV);
    row i = join/split view of A (L329-334); reading A10 (row-major). */
 void oracle_gemv(int64_t m, int64_t n, const float *A, const float *x,

@@ -66,6 +66,40 @@ def test_dot_bruteforce_fraction(n, seed):
     assert abs(Fraction(mag) - exact_mag) <= Fraction((n + 1) * EPS64 * float(exact_mag) + 1e-300)
 
 
+@pytest.mark.parametrize("n", [1, 5, 33, 64])
+def test_dot_chunked_bruteforce_and_extremes(n):
+    # the all-core dot (reading R23): Fraction brute force within the fp64 bound, and
+    # its two extreme groupings ARE the plain left fold — one chunk (the fold itself)
+    # and one element per chunk (exact products folded in order)
+    x, y = rand_f32(3, (n,)), rand_f32(4, (n,))
+    exact = sum((F(a) * F(b) for a, b in zip(x, y)), Fraction(0))
+    exact_mag = sum((abs(F(a) * F(b)) for a, b in zip(x, y)), Fraction(0))
+    s1, m1 = oracle.dot(x, y)
+    for chunks in (1, 2, 3, n):
+        s, mag = oracle.dot_chunked(x, y, chunks=chunks, threads=3)
+        assert_close_exact([s], [exact], n, [mag])
+        assert_close_exact([mag], [exact_mag], n, [mag])
+    assert oracle.dot_chunked(x, y, chunks=1)[0] == s1
+    assert oracle.dot_chunked(x, y, chunks=n)[0] == s1
+    # wide-range data, where fp64 association matters: still exactly the left fold at
+    # the two extremes (so the chunk sums are combined in chunk order)
+    xw, yw = synth.numpy_wide(5, 0, 4096, -60, 60), synth.numpy_wide(6, 0, 4096, -60, 60)
+    sw, _ = oracle.dot(xw, yw)
+    assert sw != oracle.dot(xw[::-1], yw[::-1])[0]  # the data does separate orders
+    assert oracle.dot_chunked(xw, yw, chunks=1)[0] == sw
+    assert oracle.dot_chunked(xw, yw, chunks=4096, threads=4)[0] == sw
+
+
+def test_dot_chunked_thread_invariant_and_close():
+    n = (1 << 22) + 17
+    x, y = rand_f32(0, (n,)), rand_f32(1, (n,))
+    ref = oracle.dot_chunked(x, y, chunks=256, threads=1)
+    for th in (2, 5, 16):
+        assert oracle.dot_chunked(x, y, chunks=256, threads=th) == ref
+    s, mag = oracle.dot(x, y)
+    assert abs(ref[0] - s) <= 1e-12 * mag and ref[1] == pytest.approx(mag, rel=1e-12)
+
+
 def test_dot_empty_is_zero():
     # reduceSeq(z=0, f, []) = z  (L320)
     s, mag = oracle.dot(np.zeros(0, np.float32), np.zeros(0, np.float32))

@@ -37,6 +37,10 @@ MUTATIONS = [
     ("dot_sign", "s = s + p;", "s = s - p;", 0),
     ("dot_dropped_term", "for (int64_t i = 0; i < n; ++i) {\n        double p", "for (int64_t i = 1; i < n; ++i) {\n        double p", 0),
     ("dot_mag_x100", "if (mag) *mag = a;", "if (mag) *mag = 100.0 * a;", 0),
+    # all-core dot (reading R23): a chunk boundary off by one, chunks combined in reverse
+    ("dot_chunked_boundary", "const int64_t i0 = n * k / chunks, i1 = n * (k + 1) / chunks;",
+     "const int64_t i0 = n * k / chunks, i1 = n * (k + 1) / chunks - (k == 0);", 0),
+    ("dot_chunked_reverse_combine", "        s = s + cs[k];\n", "        s = s + cs[chunks - 1 - k];\n", 0),
     # GEMV: dropped last column, mag inflated, wrong x index
     ("gemv_dropped_term", "for (int64_t j = 0; j < n; ++j) {\n            double p = (double)Ai[j] * (double)x[j];",
      "for (int64_t j = 0; j < n - 1; ++j) {\n            double p = (double)Ai[j] * (double)x[j];", 0),
