@@ -548,10 +548,12 @@ __device__ __forceinline__ void grid_barrier(unsigned int *gbar) {
             __threadfence();  // publish this block's partial row
             atomicAdd(gbar, 1u);
         }
+        // one thread per block polls the counter without back-off (a __nanosleep
+        // between polls costs ~0.3 us per launch: profiles/r02_atax_sync_ab.txt);
         // bounded: blocks that are not all resident (a concurrent kernel holding
         // SMs under a plain launch) trap after the spin limit instead of hanging
         SpinDeadline dl;
-        while (ld_acquire_gpu(gbar) < gridDim.x) dl.pause("grid barrier: not every block is resident");
+        while (ld_acquire_gpu(gbar) < gridDim.x) dl.spin("grid barrier: not every block is resident");
     }
     __syncthreads();
 }

@@ -37,14 +37,24 @@ __device__ __forceinline__ unsigned long long globaltimer_ns() {
 
 struct SpinDeadline {
     unsigned long long t0 = 0;
-    // one failed poll: back off; trap once the limit has passed since the first
-    __device__ __forceinline__ void pause(const char * /* what is awaited (documentation) */, unsigned ns = 64) {
-        __nanosleep(ns);
+    unsigned int polls = 0;
+    // trap once the limit has passed since the first call
+    __device__ __forceinline__ void check(const char * /* what is awaited (documentation) */) {
         const unsigned long long t = globaltimer_ns();
         if (t0 == 0)
             t0 = t;
         else if (t - t0 > g_spin_limit_ns)
             __trap();
+    }
+    // one failed poll: back off, then check the deadline
+    __device__ __forceinline__ void pause(const char *what, unsigned ns = 64) {
+        __nanosleep(ns);
+        check(what);
+    }
+    // one failed poll of a latency-critical wait: no back-off, the deadline
+    // checked every 256 polls
+    __device__ __forceinline__ void spin(const char *what) {
+        if ((++polls & 255u) == 0) check(what);
     }
 };
 
