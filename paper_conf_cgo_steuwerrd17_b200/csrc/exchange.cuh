@@ -104,8 +104,8 @@ __device__ __forceinline__ void exch_signal(const Exch &e, int dst /* -1: all ra
 __device__ __forceinline__ void exch_wait_all(const Exch &e, uint64_t epoch) {
     const uint64_t *f = exch_flags(e.peers[e.rank]);
     SpinDeadline dl;
-    for (int r = 0; r < e.world; ++r)
-        while (ld_acquire_sys(f + r) < epoch) dl.pause("exchange: a peer never published its data");
+    for (int r = 0; r < e.world; ++r)  // no back-off: on the critical path of every fused collective
+        while (ld_acquire_sys(f + r) < epoch) dl.spin("exchange: a peer never published its data");
 }
 
 // The last act of a call: this rank is done with `epoch` (its reads of its own
