@@ -130,12 +130,17 @@ LIFT_API int lift_gesummv(int64_t m, int64_t n, float alpha, const float *A, flo
  *                      after a grid barrier, a fixed-order reduce of the
  *                      per-block y_part (reads A once: 4*m*n bytes).
  *                      Needs 16-byte aligned A, x, y and n % 4 == 0; rows
- *                      of n <= 8192 are streamed by one block each, wider
- *                      rows (n <= 262144, n a multiple of 4C whose slices
- *                      are at most 4096 float4) by one block (n <= 16384)
- *                      or a thread-block cluster of C = 2..16 blocks over
- *                      column slices.  Other
+ *                      of n <= 16384 are streamed by one block each (one
+ *                      cooperative launch of one block per SM), wider rows
+ *                      (n <= 262144, n a multiple of 4C whose slices are at
+ *                      most 4096 float4) by a thread-block cluster of
+ *                      C = 2..16 blocks over column slices (launched
+ *                      cooperative with its cluster shape).  Other
  *                      shapes: LIFT_ERR_BAD_SIZE (auto uses TWOPASS).
+ *                      The grid barrier's wait is bounded: if the blocks
+ *                      could not all be resident it traps after the spin
+ *                      limit (LIFT_SPIN_TIMEOUT_MS, default 20 s) and the
+ *                      error surfaces at the next synchronisation.
  *   LIFT_ATAX_TWOPASS  the paper's structure (two GEMV-shaped kernels whose
  *                      times are summed, L1006-1007): GEMV t = A x, then a
  *                      column-blocked A^T t into per-row-split partials, then

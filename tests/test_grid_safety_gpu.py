@@ -66,8 +66,45 @@ def test_plain_launch_grid_barrier_fails_cleanly(hog_so):
     assert el < 60
 
 
+def test_missing_peer_fails_cleanly(hog_so):
+    """A fused collective whose peer never makes the matching call (rank 1 of a
+    simulated world of 2 never launches): rank 0's kernel waits for the peer's
+    flag only until the spin limit, then traps — a CUDA error, not a hang."""
+    r, el = run_child("peer", hog_so, 1500, 0.0)
+    assert r.returncode == 0, r.stdout + r.stderr
+    assert "failed after" in r.stdout, r.stdout
+    failed = float(r.stdout.split("failed after ")[1].split(" s")[0])
+    assert 1.0 <= failed < 15.0, r.stdout
+    assert el < 60
+
+
 # --------------------------------------------------------------------- child process
+def _peer_child():
+    import torch
+
+    import synth
+    from paper_conf_cgo_steuwerrd17_b200 import nvlink
+
+    dev = torch.device("cuda", 0)
+    n = 1 << 16
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=dev)
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_DOT, 0, 2, dev)
+    ws = torch.zeros(nvlink.workspace_bytes("dot", 0, n), dtype=torch.uint8, device=dev)
+    out = torch.empty((), device=dev)
+    torch.cuda.synchronize()
+    t1 = time.time()
+    try:
+        nvlink.lift_dot_allreduce(x, x, exs[0], out=out, workspace=ws)  # rank 1 never calls
+        torch.cuda.synchronize()
+        print(f"completed after {time.time() - t1:.2f} s (unexpected)", flush=True)
+    except Exception as e:  # noqa: BLE001
+        print(f"failed after {time.time() - t1:.2f} s: {type(e).__name__}: {str(e)[:200]}", flush=True)
+    os._exit(0)
+
+
 def _child(case, so, release_s):
+    if case == "peer":
+        _peer_child()
     import torch
 
     import oracle
