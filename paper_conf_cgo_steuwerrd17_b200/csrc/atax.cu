@@ -642,15 +642,19 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     int slot = 0;        // ring slot of stage k (k % nst), tracked without division
     uint32_t phase = 0;  // its mbarrier phase parity ((k / nst) & 1)
     int pslot = 0;       // ring slot of stage k-1
-    int64_t k = 0;
+    int k = 0;           // step (a block streams fewer than 2^31 stages)
+    // rows of every stage but the last is CR: the per-step count is two int32
+    // compares (the 64-bit stage arithmetic stays with the thread issuing copies)
+    const int nstg = (int)nstages;
+    const int last_rows = nstg > 0 ? stage_rows(nstg - 1) : 0;
     // Two register sets of CR rows: one step loads the current stage into `cur`
     // and applies the previous stage's updates from `prev`; steps alternate the
     // roles (no register copies between steps).  Returns true after the last.
     float4 ra[CR][QC], rb2[CR][QC];
     auto step = [&](float4(&cur)[CR][QC], float4(&prev)[CR][QC]) -> bool {
-        const int rows = stage_rows(k);
+        const int rows = k < nstg - 1 ? CR : (k == nstg - 1 ? last_rows : 0);
         __syncthreads();  // previous stage: partials published, slot consumed
-        if (tid == 0 && prow > 0 && k - 1 + nst < nstages) issue_stage(k - 1 + nst, pslot);
+        if (tid == 0 && prow > 0 && k - 1 + nst < nstg) issue_stage(k - 1 + nst, pslot);
         float *rb = red + buf * CR * kFusedWarps;
         if (rows > 0) {
             mbar_wait_parity(full + slot, phase);
