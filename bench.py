@@ -682,6 +682,7 @@ def run_ours(args) -> None:
                      "ms_min": round(op_min_ms[name], 4) if name in op_min_ms else None,
                      "alg_bytes": by, "GB_s": round(gbs, 1),
                      "frac_of_peak_per_gpu": round(gbs / world / peak, 4),
+                     "frac_of_spec_peak_per_gpu": round(gbs / world / spec_peak(), 4),
                      "ncu_dram_pct_of_peak": load_ncu(kern, name).get("ncu_dram_pct_of_peak")}
     # N > 1: each op's local kernel alone (no collective), so the JSON line separates
     # compute-only per-rank GB/s from the collective's time (max over ranks, like `ms`)
@@ -798,6 +799,10 @@ def run_ours(args) -> None:
                                  else "eager",
                        "frac_of_peak_per_gpu": round(value / world / peak, 4)},
             "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": gpu_launches,
+            # the step's GB/s is dominated by the two largest ops: name the weakest op too
+            "ops_weakest": min(({"op": k, "GB_s": v["GB_s"], "frac_of_spec_peak_per_gpu":
+                                 v["frac_of_spec_peak_per_gpu"], "ncu_dram_pct_of_peak": v["ncu_dram_pct_of_peak"]}
+                                for k, v in ops.items()), key=lambda d: d["frac_of_spec_peak_per_gpu"]),
             "clocks": sampler.summary(), "ops": ops, "table1": table1,
             "table1_method": "the paper's small/large sizes (Table 1) and configs[0]: >= 20 back-to-back calls "
                              "in one CUDA graph after the timed region, operands rotated over slices totalling "
