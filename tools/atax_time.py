@@ -27,6 +27,8 @@ for m, n in shapes:
     got = lift.lift_atax(As[0], x, algo="fused").cpu().numpy()
     ok, margin = oracle.within_tol(got, *oracle.atax(As[0].cpu().numpy(), x.cpu().numpy()))
     t = graph_time([(lambda A=A: lift.lift_atax(A, x, out=y, algo="fused")) for A in (As * 24)[:24]])
-    print(f"atax {m}x{n}: {t:8.2f} us  {4 * m * n / t / 1e3:8.1f} GB/s  parity {'ok' if ok else 'BAD'} {margin:.2g}",
-          flush=True)
+    import zlib
+    crc = zlib.crc32(got.view("uint32").tobytes())  # compare the exact bits across builds / settings
+    print(f"atax {m}x{n}: {t:8.2f} us  {4 * m * n / t / 1e3:8.1f} GB/s  parity {'ok' if ok else 'BAD'} {margin:.2g}"
+          f"  bits {crc:08x}", flush=True)
     del As
