@@ -609,14 +609,9 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     __syncthreads();
     if (tid == 0)  // prologue: fill the ring
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
-    // fused (all-)reduce: this call's epoch; the destinations have finished with
-    // the parity buffer this call writes (checked now, while the ring fills; the
-    // main loop's first block barrier orders the later pushes after it)
-    uint64_t ep = 0;
-    if (ex.world > 0) {
-        ep = exch_epoch(ex);
-        if (tid == 0) exch_wait_consumed_all(ex, dst, ep);
-    }
+    // fused (all-)reduce: this call's epoch (its parity buffer is free: the previous
+    // call's exch_finish saw every destination done with it)
+    const uint64_t ep = ex.world > 0 ? exch_epoch(ex) : 0ull;
 
     constexpr bool XS = QC >= kFusedXsmemQc;  // x in shared memory (after the ring) instead of registers
     float4 xr[XS ? 1 : QC], yr[QC];
@@ -752,15 +747,16 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     __syncthreads();
     __shared__ int last_block;
     if (threadIdx.x == 0) {
-        __threadfence_system();
-        const unsigned int dep = atomicAdd(gbar + 1, 1u) + 1u;
+        // gpu-scope release of this block's pushes; the last block acquires them all and
+        // releases to the destination(s) at system scope once (exchange.cuh)
+        const unsigned int dep = atom_acq_rel_add(gbar + 1, 1u) + 1u;
         last_block = dep == gridDim.x;
         if (last_block) {  // every block has pushed (and passed the grid barrier): re-arm, publish
             gbar[0] = 0u;
             gbar[1] = 0u;
             exch_signal(ex, dst, ep);
             // a rank that receives nothing is done with this epoch once it has published
-            if (dst >= 0 && ex.rank != dst) exch_ack(ex, ep);
+            if (dst >= 0 && ex.rank != dst) exch_finish(ex, ep);
         }
     }
     if (dst >= 0 && ex.rank != dst) return;
@@ -769,12 +765,12 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     const float *src = exch_data(ex.peers[ex.rank], ex, ep);
     for (int64_t c = c0 + threadIdx.x; c < c1; c += blockDim.x) {
         float4 acc = zero4();
-        for (int r = 0; r < ex.world; ++r) {
-            const float *p = src + (int64_t)r * n + 4 * c;
-            acc.x = __fadd_rn(acc.x, ld_volatile(p));
-            acc.y = __fadd_rn(acc.y, ld_volatile(p + 1));
-            acc.z = __fadd_rn(acc.z, ld_volatile(p + 2));
-            acc.w = __fadd_rn(acc.w, ld_volatile(p + 3));
+        for (int r = 0; r < ex.world; ++r) {  // rank order; L2 loads after thread 0's acquire + the barrier
+            const float4 v = __ldcg(reinterpret_cast<const float4 *>(src + (int64_t)r * n) + c);
+            acc.x = __fadd_rn(acc.x, v.x);
+            acc.y = __fadd_rn(acc.y, v.y);
+            acc.z = __fadd_rn(acc.z, v.z);
+            acc.w = __fadd_rn(acc.w, v.w);
         }
         reinterpret_cast<float4 *>(y)[c] = acc;
     }
@@ -785,7 +781,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         unsigned int *readers = exch_readers(ex.peers[ex.rank]);
         if (atom_acq_rel_add(readers, 1u) == gridDim.x - 1) {
             *readers = 0u;
-            exch_ack(ex, ep);
+            exch_finish(ex, ep);
         }
     }
 }

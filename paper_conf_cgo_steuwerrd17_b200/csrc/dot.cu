@@ -127,16 +127,14 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
             // rank's exchange area, publish, wait for all ranks, then every rank sums
             // the slots in rank order: bitwise identical results on all ranks
             const uint64_t ep = exch_epoch(ex);
-            exch_wait_consumed_all(ex, -1, ep);
             for (int q = 0; q < ex.world; ++q) exch_data(ex.peers[q], ex, ep)[ex.rank] = tot;
-            __threadfence_system();
-            exch_signal(ex, -1, ep);
+            exch_signal(ex, -1, ep);  // st.release.sys: the slot stores above first
             exch_wait_all(ex, ep);
             const float *d = exch_data(ex.peers[ex.rank], ex, ep);
             float sum = 0.f;
             for (int r = 0; r < ex.world; ++r) sum = __fadd_rn(sum, ld_volatile(d + r));
             *result = sum;
-            exch_ack(ex, ep);
+            exch_finish(ex, ep);
         }
     }
 }

@@ -21,12 +21,34 @@
 // in a CUDA graph and replayed.
 //
 // Buffer reuse: the data of epoch e goes to parity e & 1, last used by epoch
-// e - 2.  Before rank p stores epoch e's data into rank q's area it waits
-// until ack[q] (in p's OWN area, written there by q) >= e - 2, i.e. q has
-// finished reading epoch e - 2.  This holds in every mode — all-gather,
-// all-reduce and reduce-to-one-rank, where the senders do not wait for the
-// destination and could otherwise run two calls ahead — and in any mix of
-// them.  The check is a local load, normally satisfied at the first read.
+// e - 2.  A rank may store epoch e's data into rank q's area only once q has
+// finished reading epoch e - 2, i.e. ack[q] (in the writer's OWN area, written
+// there by q) >= e - 2.  The check runs at the END of the previous call:
+// after acknowledging epoch e - 1, a rank's last block waits until every
+// rank's ack >= e - 2, before the kernel completes — so the next call's
+// kernels, which start after it, never need it.  This holds in every mode —
+// all-gather, all-reduce and reduce-to-one-rank, where the senders do not
+// wait for the destination and could otherwise run two calls ahead — and in
+// any mix of them.  It is a local load, normally satisfied at the first read
+// (in the all-modes the flags of epoch e - 1 already imply it).
+//
+// Memory ordering, with as few system-scope operations as possible (a
+// system-scope fence costs microseconds): the blocks of a kernel publish
+// their stores into the exchange areas to ONE block of their GPU with
+// gpu-scope acquire-release atomics (a ticket); that last block then releases
+// at system scope (st.release.sys of the flags).  Causality is transitive in
+// the PTX memory model (gpu-scope synchronisation inside the GPU, system scope
+// from that block to the peers), so a peer that acquires the flag
+// (ld.acquire.sys) sees every block's data.  No fence.sc / fence.acq_rel.sys
+// anywhere: they measured slower than the release / acquire accesses
+// (tools/fused_overhead.py, profiles/r02_fused_epilogue_ab.txt).
+//
+// The acknowledgements guard a write-after-read hazard only (a sender must not
+// overwrite data a peer has not read yet), so they are relaxed accesses, the
+// way NCCL's flag protocols treat the same hazard: a rank writes its ack after
+// it has consumed the values it read (they fed the sums it stored), and a
+// sender's next stores come after its check observed the ack (in a later
+// kernel on the same stream).
 #pragma once
 
 #include <stdint.h>
@@ -68,6 +90,10 @@ __device__ __forceinline__ uint64_t ld_relaxed_sys(const uint64_t *p) {
     asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
     return v;
 }
+__device__ __forceinline__ void st_relaxed_sys(uint64_t *p, uint64_t v) {
+    asm volatile("st.relaxed.sys.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ void fence_acq_rel_sys() { asm volatile("fence.acq_rel.sys;" ::: "memory"); }
 __device__ __forceinline__ float ld_volatile(const float *p) {
     float v;
     asm volatile("ld.volatile.global.f32 %0, [%1];" : "=f"(v) : "l"(p) : "memory");
@@ -79,19 +105,8 @@ __device__ __forceinline__ uint64_t exch_epoch(const Exch &e) {
     return ld_relaxed_sys(exch_acks(e.peers[e.rank]) + e.rank) + 1ull;
 }
 
-// Before storing epoch `epoch`'s data into rank q's area: q has finished with
-// epoch - 2 (the last user of this parity buffer).  Bounded like every spin.
-__device__ __forceinline__ void exch_wait_consumed(const Exch &e, int q, uint64_t epoch) {
-    const uint64_t *a = exch_acks(e.peers[e.rank]) + q;
-    SpinDeadline dl;
-    while (ld_acquire_sys(a) + 2ull < epoch) dl.pause("exchange: peer never consumed an earlier epoch");
-}
-__device__ __forceinline__ void exch_wait_consumed_all(const Exch &e, int dst /* -1: all ranks */, uint64_t epoch) {
-    for (int q = 0; q < e.world; ++q)
-        if (dst < 0 || q == dst) exch_wait_consumed(e, q, epoch);
-}
-
-// After this rank's data stores to the peers: publish (caller did fence.sys).
+// After this rank's data stores to the peers (this thread's own, and every
+// other block's, acquired through a gpu-scope ticket): publish, one release.
 __device__ __forceinline__ void exch_signal(const Exch &e, int dst /* -1: all ranks */, uint64_t epoch) {
     for (int p = 0; p < e.world; ++p)
         if (dst < 0 || p == dst) st_release_sys(exch_flags(e.peers[p]) + e.rank, epoch);
@@ -108,11 +123,17 @@ __device__ __forceinline__ void exch_wait_all(const Exch &e, uint64_t epoch) {
         while (ld_acquire_sys(f + r) < epoch) dl.spin("exchange: a peer never published its data");
 }
 
-// The last act of a call: this rank is done with `epoch` (its reads of its own
-// area are complete).  Written into every rank's area; the own copy is also
-// the next call's epoch base.
-__device__ __forceinline__ void exch_ack(const Exch &e, uint64_t epoch) {
-    for (int p = 0; p < e.world; ++p) st_release_sys(exch_acks(e.peers[p]) + e.rank, epoch);
+// The last act of a call (one thread of the last block): this rank is done
+// with `epoch` (its reads of its own area are complete and consumed) — written
+// into every rank's area (relaxed: see above; the own copy is also the next
+// call's epoch base) — and, for the NEXT call's stores, every rank has
+// finished `epoch` - 1, whose parity buffer that call writes.  Bounded.
+__device__ __forceinline__ void exch_finish(const Exch &e, uint64_t epoch) {
+    for (int p = 0; p < e.world; ++p) st_relaxed_sys(exch_acks(e.peers[p]) + e.rank, epoch);
+    const uint64_t *a = exch_acks(e.peers[e.rank]);
+    SpinDeadline dl;
+    for (int q = 0; q < e.world; ++q)
+        while (ld_relaxed_sys(a + q) + 1ull < epoch) dl.pause("exchange: a peer never finished an earlier call");
 }
 
 }  // namespace lift

@@ -86,15 +86,12 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     const int64_t kfull = nv / kVLanes;                   // k-steps whose every vector is in the row
     const int lane_off = kWarp * (wr * KQ) + lane;        // first virtual lane of this lane, slice q adds 32*q
 
-    // fused all-gather: this call's epoch, and every destination has finished
-    // with the parity buffer this call writes (the barrier orders the row
-    // writers after the check)
+    // fused all-gather: this call's epoch (its parity buffer is free: the previous
+    // call's exch_finish saw every destination done with it).  The exchange stays
+    // a runtime branch of the one kernel: a separate template instantiation
+    // without it compiled the plain GEMV 9 % slower (profiles/r02_fused_epilogue_ab.txt).
     uint64_t ep = 0;
-    if (ex.world > 0) {
-        ep = exch_epoch(ex);
-        if (threadIdx.x == 0) exch_wait_consumed_all(ex, -1, ep);
-        __syncthreads();
-    }
+    if (ex.world > 0) ep = exch_epoch(ex);
     bool x_pending = false;
     if constexpr (XSMEM) {
         stage_issue(xs, x, (uint32_t)(n * 4), bar);  // toLocal(x), one bulk copy per block
@@ -260,10 +257,9 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
         // waits for every rank, then copies the gathered y out of the exchange area
         __shared__ int am_last;
         __syncthreads();
-        if (threadIdx.x == 0) {
-            __threadfence_system();  // this block's remote row stores are visible system-wide
-            am_last = atomicAdd(ticket, 1u) == gridDim.x - 1;
-        }
+        if (threadIdx.x == 0)  // gpu-scope release of this block's row stores; the last block
+            // acquires them all and releases to the peers at system scope once (exchange.cuh)
+            am_last = atom_acq_rel_add(ticket, 1u) == gridDim.x - 1;
         __syncthreads();
         if (!am_last) return;
         if (threadIdx.x == 0) {
@@ -272,10 +268,12 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
             exch_wait_all(ex, ep);
         }
         __syncthreads();
+        // the gathered rows, after thread 0's acquire of every rank's flag and the barrier:
+        // L2 loads (no stale L1 line)
         const float *src = exch_data(ex.peers[ex.rank], ex, ep);
-        for (int64_t i = threadIdx.x; i < m_total; i += blockDim.x) y[i] = ld_volatile(src + i);
+        for (int64_t i = threadIdx.x; i < m_total; i += blockDim.x) y[i] = __ldcg(src + i);
         __syncthreads();  // every read of this epoch's data is done
-        if (threadIdx.x == 0) exch_ack(ex, ep);
+        if (threadIdx.x == 0) exch_finish(ex, ep);
     }
 }
 

@@ -14,8 +14,9 @@ import sys
 
 import torch
 
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 sys.path.insert(0, os.path.dirname(os.path.abspath(__file__)))
+# LIFT_ROOT: the package root to time (tools/ab_tree.sh points it at an older tree)
+sys.path.insert(0, os.environ.get("LIFT_ROOT") or os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import synth  # noqa: E402
 import paper_conf_cgo_steuwerrd17_b200 as lift  # noqa: E402
 
