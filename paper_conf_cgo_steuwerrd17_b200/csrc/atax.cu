@@ -120,6 +120,7 @@ __global__ void __launch_bounds__(kColsumWarps * 32) k_colsum(int S, int64_t nv,
                                                                 float *__restrict__ y, float alpha, float beta,
                                                                 bool axpby) {
     __shared__ __align__(16) float part[kColsumWarps * 32 * VEC];
+    pdl_wait_and_release();
     colsum_tile<VEC, kColsumWarps>(S, nv, P, y, (int64_t)blockIdx.x * 32, part, alpha, beta, axpby);
 }
 
@@ -128,8 +129,8 @@ static cudaError_t run_colsum(int S, int64_t n, const float *P, float *y, cudaSt
                               float beta = 0.f, bool axpby = false) {
     const int64_t nv = n / VEC;
     const int64_t blocks = (nv + 31) / 32;
-    k_colsum<VEC><<<(unsigned)blocks, kColsumWarps * 32, 0, s>>>(S, nv, P, y, alpha, beta, axpby);
-    return cudaGetLastError();
+    return launch_pdl(k_colsum<VEC>, dim3((unsigned)blocks), dim3(kColsumWarps * 32), 0, s, S, nv, P, y, alpha, beta,
+                      axpby);
 }
 
 // ---------------------------------------------------------------------------
@@ -140,6 +141,7 @@ __global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int64_t
                                                    const float *__restrict__ A, const float *__restrict__ t,
                                                    float *__restrict__ P) {
     using V = typename std::conditional<VEC == 4, float4, float>::type;
+    pdl_wait_and_release();
     const int s = blockIdx.y;
     const int64_t r0 = m * s / S, r1 = m * (s + 1) / S;
     const int64_t nv = n / VEC;
@@ -205,11 +207,8 @@ static cudaError_t column_pass(const DeviceInfo &d, int64_t m, int64_t n, int64_
     if (S > m) S = m;
     if (S < 1) S = 1;
     dim3 grid((unsigned)cblocks, (unsigned)S);
-    if (vec)
-        k_atax_cols<4, TPB, 8><<<grid, TPB, 0, s>>>(m, n, lda, (int)S, A, t, P);
-    else
-        k_atax_cols<1, TPB, 8><<<grid, TPB, 0, s>>>(m, n, lda, (int)S, A, t, P);
-    e = cudaGetLastError();
+    e = vec ? launch_pdl(k_atax_cols<4, TPB, 8>, grid, dim3(TPB), 0, s, m, n, lda, (int)S, A, t, P)
+            : launch_pdl(k_atax_cols<1, TPB, 8>, grid, dim3(TPB), 0, s, m, n, lda, (int)S, A, t, P);
     if (e != cudaSuccess) return e;
     return vec ? run_colsum<4>((int)S, n, P, y, s, alpha, beta, axpby)
                : run_colsum<1>((int)S, n, P, y, s, alpha, beta, axpby);

@@ -128,6 +128,43 @@ static inline cudaError_t ensure_smem(K kern, int dev, size_t smem) {
 }
 
 // ---------------------------------------------------------------------------
+// Programmatic dependent launch (PDL): the streaming kernels are launched with
+// cudaLaunchAttributeProgrammaticStreamSerialization, so the next kernel on the
+// stream can be scheduled onto SMs as this one's blocks retire; each kernel
+// starts with griddepcontrol.wait (before ANY global memory access: the
+// previous kernel may produce its inputs or read its outputs) and then lets
+// its own dependent launch.  The cooperative fused ATAX is launched plainly.
+// LIFT_PDL=0 turns it off (A/B).
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ void pdl_wait_and_release() {
+    asm volatile("griddepcontrol.wait;" ::: "memory");
+    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+}
+static inline bool pdl_enabled() {
+    static const bool on = [] {
+        const char *v = getenv("LIFT_PDL");
+        return !(v && v[0] == '0');
+    }();
+    return on;
+}
+// kern<<<grid, block, smem, s>>>(args...) with the PDL attribute
+template <typename... KArgs, typename... Args>
+static inline cudaError_t launch_pdl(void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t s,
+                                     Args &&...args) {
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    attr[0].val.programmaticStreamSerializationAllowed = pdl_enabled() ? 1 : 0;
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = s;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelEx(&cfg, kern, static_cast<KArgs>(args)...);
+}
+
+// ---------------------------------------------------------------------------
 // Global loads
 // ---------------------------------------------------------------------------
 
