@@ -128,6 +128,7 @@ def _launch_sequence(world, calls, delay_rank=None, delay_cycles=0):
     `delay_rank`'s stream sleeps before each of its calls, so the other ranks run
     ahead of it as far as the protocol lets them."""
     streams = [torch.cuda.Stream() for _ in range(world)]
+    torch.cuda._sleep(1)  # load torch's sleep kernel now: a lazy module load waits for an idle device
     torch.cuda.synchronize()
     for k in range(len(calls)):
         for r in range(world):
@@ -193,3 +194,64 @@ def test_mixed_collectives_back_to_back_no_sync(cuda_device, world):
             for r in (range(world) if modes[k] < 0 else [modes[k]]):
                 ok, margin = oracle.within_tol(outs[k][r].cpu().numpy(), ref, mag)
                 assert ok, (delayed, k, r, margin)
+
+
+@pytest.mark.parametrize("seed", [1, 2, 3])
+def test_exchange_random_sequences_no_sync(cuda_device, seed):
+    """Random sequences of fused calls on simulated ranks, every rank issuing its
+    calls back to back with no host synchronisation, a random rank's stream
+    delayed by a random amount before each call: ATAX reductions with random
+    destinations (-1 = all) on one exchange area and dot all-reduces on another,
+    interleaved.  Every call's result must be that call's own (different x per
+    call), so no run-ahead or parity mix-up goes unnoticed."""
+    rng = np.random.default_rng(seed)
+    world = int(rng.integers(2, 5))
+    m, n = 300, 512
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    K = 10
+    xs = [synth.torch_uniform(300 + 17 * seed + k, 0, n, device=cuda_device) for k in range(K)]
+    nd = 4096 + int(rng.integers(0, 100))
+    dvs = [synth.torch_uniform(500 + 17 * seed + k, 0, nd, device=cuda_device) for k in range(K)]
+    ex_a = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, world, cuda_device)
+    ex_d = nvlink.ExchangeArea.simulated(nvlink.EXCH_DOT, 0, world, cuda_device)
+    parts = [partition_rows(m, world, r) for r in range(world)]
+    dparts = [partition_rows(nd, world, r) for r in range(world)]
+    ws_a = [torch.zeros(nvlink.workspace_bytes("atax", m, n), dtype=torch.uint8, device=cuda_device)
+            for _ in range(world)]
+    ws_d = [torch.zeros(nvlink.workspace_bytes("dot", 0, nd), dtype=torch.uint8, device=cuda_device)
+            for _ in range(world)]
+    kinds = rng.integers(0, 2, K)  # 0: ATAX reduce, 1: dot all-reduce
+    dsts = rng.integers(-1, world, K)
+    delays = [(int(rng.integers(0, world)), int(rng.integers(0, 400_000))) for _ in range(K)]
+    outs = [[torch.full((n,) if kinds[k] == 0 else (), float("nan"), device=cuda_device) for _ in range(world)]
+            for k in range(K)]
+    blocks = 148 // (world + 1)
+    streams = [torch.cuda.Stream() for _ in range(world)]
+    torch.cuda._sleep(1)  # load torch's sleep kernel now: a lazy module load waits for an idle device,
+    torch.cuda.synchronize()  # which ranks spinning on each other's flags never leave
+    for k in range(K):
+        for r in range(world):
+            with torch.cuda.stream(streams[r]):
+                if r == delays[k][0]:
+                    torch.cuda._sleep(delays[k][1])
+                if kinds[k] == 0:
+                    nvlink.lift_atax_reduce(A[parts[r][0]:parts[r][1]], xs[k], ex_a[r], dst=int(dsts[k]),
+                                            blocks=blocks, out=outs[k][r], workspace=ws_a[r])
+                else:
+                    a, b = dparts[r]
+                    nvlink.lift_dot_allreduce(dvs[k][a:b], dvs[k][a:b], ex_d[r], out=outs[k][r], workspace=ws_d[r])
+    torch.cuda.synchronize()
+    An = A.cpu().numpy()
+    for k in range(K):
+        if kinds[k] == 0:
+            ref, mag = oracle.atax(An, xs[k].cpu().numpy())
+            for r in (range(world) if dsts[k] < 0 else [int(dsts[k])]):
+                ok, margin = oracle.within_tol(outs[k][r].cpu().numpy(), ref, mag)
+                assert ok, (seed, k, r, margin)
+        else:
+            v = dvs[k].cpu().numpy()
+            ref, mag = oracle.dot(v, v)
+            vals = [outs[k][r].item() for r in range(world)]
+            assert all(np.float32(a).view(np.uint32) == np.float32(vals[0]).view(np.uint32) for a in vals), (k, vals)
+            ok, margin = oracle.within_tol([vals[0]], [ref], [mag])
+            assert ok, (seed, k, margin)
