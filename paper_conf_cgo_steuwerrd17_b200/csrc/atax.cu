@@ -129,7 +129,7 @@ static cudaError_t run_colsum(int S, int64_t n, const float *P, float *y, cudaSt
                               float beta = 0.f, bool axpby = false) {
     const int64_t nv = n / VEC;
     const int64_t blocks = (nv + 31) / 32;
-    return launch_pdl(k_colsum<VEC>, dim3((unsigned)blocks), dim3(kColsumWarps * 32), 0, s, S, nv, P, y, alpha, beta,
+    return launch_pdl(true, k_colsum<VEC>, dim3((unsigned)blocks), dim3(kColsumWarps * 32), 0, s, S, nv, P, y, alpha, beta,
                       axpby);
 }
 
@@ -207,8 +207,8 @@ static cudaError_t column_pass(const DeviceInfo &d, int64_t m, int64_t n, int64_
     if (S > m) S = m;
     if (S < 1) S = 1;
     dim3 grid((unsigned)cblocks, (unsigned)S);
-    e = vec ? launch_pdl(k_atax_cols<4, TPB, 8>, grid, dim3(TPB), 0, s, m, n, lda, (int)S, A, t, P)
-            : launch_pdl(k_atax_cols<1, TPB, 8>, grid, dim3(TPB), 0, s, m, n, lda, (int)S, A, t, P);
+    e = vec ? launch_pdl(true, k_atax_cols<4, TPB, 8>, grid, dim3(TPB), 0, s, m, n, lda, (int)S, A, t, P)
+            : launch_pdl(true, k_atax_cols<1, TPB, 8>, grid, dim3(TPB), 0, s, m, n, lda, (int)S, A, t, P);
     if (e != cudaSuccess) return e;
     return vec ? run_colsum<4>((int)S, n, P, y, s, alpha, beta, axpby)
                : run_colsum<1>((int)S, n, P, y, s, alpha, beta, axpby);

@@ -136,9 +136,11 @@ static inline cudaError_t ensure_smem(K kern, int dev, size_t smem) {
 // its own dependent launch.  The cooperative fused ATAX is launched plainly.
 // LIFT_PDL=0 turns it off (A/B).
 // ---------------------------------------------------------------------------
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void pdl_release() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
 __device__ __forceinline__ void pdl_wait_and_release() {
-    asm volatile("griddepcontrol.wait;" ::: "memory");
-    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+    pdl_wait();
+    pdl_release();
 }
 static inline bool pdl_enabled() {
     static const bool on = [] {
@@ -147,13 +149,15 @@ static inline bool pdl_enabled() {
     }();
     return on;
 }
-// kern<<<grid, block, smem, s>>>(args...) with the PDL attribute
+// kern<<<grid, block, smem, s>>>(args...) with the PDL attribute (unless `allow` is
+// false: the fused collectives launch plainly — a dependent's early blocks could
+// take SM slots a peer rank SHARING the GPU needs before this kernel can finish)
 template <typename... KArgs, typename... Args>
-static inline cudaError_t launch_pdl(void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t s,
-                                     Args &&...args) {
+static inline cudaError_t launch_pdl(bool allow, void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem,
+                                     cudaStream_t s, Args &&...args) {
     cudaLaunchAttribute attr[1];
     attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
-    attr[0].val.programmaticStreamSerializationAllowed = pdl_enabled() ? 1 : 0;
+    attr[0].val.programmaticStreamSerializationAllowed = (allow && pdl_enabled()) ? 1 : 0;
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = grid;
     cfg.blockDim = block;

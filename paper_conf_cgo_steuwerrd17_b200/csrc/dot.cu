@@ -40,7 +40,8 @@ __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict_
                                              unsigned int *__restrict__ ticket, Exch ex) {
     __shared__ float red[TPB / kWarp];
     __shared__ bool am_last;
-    pdl_wait_and_release();
+    pdl_wait();
+    if (ex.world == 0) pdl_release();  // a fused collective lets nothing start early beside it
     const int64_t stride = (int64_t)gridDim.x * TPB;
     int64_t i = (int64_t)blockIdx.x * TPB + threadIdx.x;
     float s;
@@ -173,8 +174,8 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     int64_t cap = (int64_t)d.sms * per_sm * (units < kOneWaveUnits ? 1 : kWaves);
     if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;
     int blocks = (int)(want < 1 ? 1 : (want > cap ? cap : want));
-    if (vec) return launch_pdl(k_dot<TPB, U, true>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex);
-    return launch_pdl(k_dot<TPB, U, false>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex);
+    if (vec) return launch_pdl(ex.world == 0, k_dot<TPB, U, true>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex);
+    return launch_pdl(ex.world == 0, k_dot<TPB, U, false>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex);
 }
 
 // Load every kernel of this unit now (CUDA's lazy loading would otherwise load a

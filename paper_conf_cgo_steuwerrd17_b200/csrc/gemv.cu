@@ -78,7 +78,8 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     float *red = reinterpret_cast<float *>(smem + 16);
     float *xs = reinterpret_cast<float *>(smem + gemv_x_offset<NMAT, RG>());
 
-    pdl_wait_and_release();
+    pdl_wait();
+    if (ex.world == 0) pdl_release();  // a fused collective lets nothing start early beside it
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int g = warp / WPR;   // row group inside the block
     const int wr = warp % WPR;  // warp rank inside the row group
@@ -300,7 +301,7 @@ static cudaError_t run_gemv(const DeviceInfo &d, const GemvArgs &a, int blocks, 
     if (groups >= 32 * cap) cap *= 4;
     int64_t g = blocks > 0 ? blocks : (groups < cap ? groups : cap);
     if (g < 1) g = 1;
-    return launch_pdl(kern, dim3((unsigned)g), dim3(threads), smem, s, a.m, a.n, a.lda, a.A, a.B, a.x, a.y, a.alpha,
+    return launch_pdl(a.ex.world == 0, kern, dim3((unsigned)g), dim3(threads), smem, s, a.m, a.n, a.lda, a.A, a.B, a.x, a.y, a.alpha,
                       a.beta, a.epi, a.ex, a.row0, a.m_total, a.ticket);
 }
 
