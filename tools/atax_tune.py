@@ -1,4 +1,6 @@
-"""Fused-ATAX ring depth x L2 prefetch distance sweep (lift_atax_fused_tuned).
+"""Fused-ATAX ring depth x row assignment sweep (lift_atax_fused_tuned).
+(Round 1 also swept an L2 bulk-prefetch distance, since removed from the
+library: profiles/r01r_atax_tune.txt.)
 
 Each timed call reads a different copy of A (copies totalling > 2x L2), so
 every call streams A from HBM; time per call from a CUDA graph of 12 calls.
@@ -23,22 +25,20 @@ for m, n, sets in shapes:
     x = synth.torch_uniform(0, 0, n, device=dev)
     y = torch.empty(n, device=dev)
     ref = lift.lift_atax(As[0], x, algo="fused").clone()
-    grid = [(nst, l2a, cyc) for cyc in (0, 1) for nst in (0, 2, 3, 4, 5, 6) for l2a in (0, 1, 2, 4)]
+    grid = [(nst, cyc) for cyc in (0, 1) for nst in (0, 2, 3, 4, 5, 6)]
     if quick:
-        grid = [(nst, 0, cyc) for cyc in (0, 1) for nst in (0, 3, 4)]
-    for nst, l2a, cyc in grid:
+        grid = [(nst, cyc) for cyc in (0, 1) for nst in (0, 3, 4)]
+    for nst, cyc in grid:
         try:
-            got = lift.lift_atax_fused_tuned(As[0], x, nst=nst, l2_ahead=l2a, cyclic=cyc)
+            got = lift.lift_atax_fused_tuned(As[0], x, nst=nst, cyclic=cyc)
         except lift.LiftError as e:
-            print(f"atax {m}x{n} cyc {cyc} nst {nst} l2a {l2a}: {e}", flush=True)
+            print(f"atax {m}x{n} cyc {cyc} nst {nst}: {e}", flush=True)
             continue
-        if cyc == 0:
-            assert torch.equal(got, ref), (nst, l2a)
+        if cyc == 1:  # the automatic assignment: bitwise the library call for every ring depth
+            assert torch.equal(got, ref), nst
         else:
-            assert torch.allclose(got, ref, rtol=1e-4, atol=1e-3), (nst, l2a)
-        calls = [(lambda A=A: lift.lift_atax_fused_tuned(A, x, out=y, nst=nst, l2_ahead=l2a, cyclic=cyc))
-                 for A in (As * 12)[:12]]
+            assert torch.allclose(got, ref, rtol=1e-4, atol=1e-3), nst
+        calls = [(lambda A=A: lift.lift_atax_fused_tuned(A, x, out=y, nst=nst, cyclic=cyc)) for A in (As * 12)[:12]]
         t = graph_time(calls)
-        print(f"atax {m}x{n} cyc {cyc} nst {nst} l2a {l2a}: {t:8.2f} us  {4 * m * n / t / 1e3:8.1f} GB/s",
-              flush=True)
+        print(f"atax {m}x{n} cyc {cyc} nst {nst}: {t:8.2f} us  {4 * m * n / t / 1e3:8.1f} GB/s", flush=True)
     del As
