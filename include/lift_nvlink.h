@@ -18,10 +18,10 @@
  * (every rank makes the matching call).  The call counter (epoch) lives in
  * the area on the device — the host passes none — so a sequence of these
  * calls can be captured in a CUDA graph and replayed.  Data is double
- * buffered by epoch parity; before a rank stores into a peer's buffer it
- * waits (on the device) until that peer has acknowledged consuming the
- * call two epochs back, so no rank overwrites data a slower rank is still
- * reading, in any mix of all-reduce, all-gather and reduce-to-one-rank calls.
+ * buffered by epoch parity; every call ends (on the device) only once every
+ * rank has acknowledged reading the previous call's data, so the next call
+ * never overwrites data a slower rank is still reading, in any mix of
+ * all-reduce, all-gather and reduce-to-one-rank calls.
  * A rank that never makes the matching call makes its peers trap after the
  * spin limit (LIFT_SPIN_TIMEOUT_MS, default 20 s; the launch fails with a
  * CUDA error at the next synchronisation) instead of hanging the GPU.
