@@ -1011,12 +1011,18 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
     // together with the cluster shape (the launch then fails instead of running a
     // grid that cannot be co-resident).  Where the driver refuses the combination
     // the launch is plain and the barrier's bounded spin is the backstop.
+    // LIFT_WIDE_COOPERATIVE=0 launches plainly (a profiling aid: ncu cannot replay the
+    // cooperative cluster launch — the kernel's waits time out under it).
     static int coop_ok[64];  // per device: 0 unknown, 1 accepted, -1 refused
+    static const bool coop_env = [] {
+        const char *v = getenv("LIFT_WIDE_COOPERATIVE");
+        return !(v && v[0] == '0');
+    }();
     cudaLaunchAttribute attr2[2] = {attr[0], {}};
     attr2[1].id = cudaLaunchAttributeCooperative;
     attr2[1].val.cooperative = 1;
     const int dev = d.device >= 0 && d.device < 64 ? d.device : 0;
-    if (coop_ok[dev] >= 0) {
+    if (coop_env && coop_ok[dev] >= 0) {
         cfg.attrs = attr2;
         cfg.numAttrs = 2;
         cudaError_t e2 = cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
