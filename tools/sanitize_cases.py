@@ -37,7 +37,8 @@ for m, n in ((7, 3), (5, 129), (33, 4096), (3, 1000), (9, 8192), (2, 20000)):
     ref, mag = oracle.atax(A, x)
     for algo in ("auto", "twopass") + (("fused",) if n % 4 == 0 and n <= 16384 else ()):
         chk(f"atax{m}x{n}{algo}", lift.lift_atax(t(A), t(x), algo=algo).cpu().numpy(), ref, mag)
-for m, n in ((40, 32), (200, 4096), (300, 8192)):
+# (600 x 12288, 7 x 8196: 8 float4 columns per thread with x in shared memory, ragged slices)
+for m, n in ((40, 32), (200, 4096), (300, 8192), (600, 12288), (7, 8196)):
     A = synth.numpy_matrix_rows(2, n, 0, m)
     x = synth.numpy_uniform(0, 0, n)
     chk(f"atax-fused{m}x{n}", lift.lift_atax(t(A), t(x), algo="fused").cpu().numpy(), *oracle.atax(A, x))
