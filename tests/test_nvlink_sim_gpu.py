@@ -255,3 +255,40 @@ def test_exchange_random_sequences_no_sync(cuda_device, seed):
             assert all(np.float32(a).view(np.uint32) == np.float32(vals[0]).view(np.uint32) for a in vals), (k, vals)
             ok, margin = oracle.within_tol([vals[0]], [ref], [mag])
             assert ok, (seed, k, margin)
+
+
+@pytest.mark.parametrize("op", ["gemv", "gesummv", "dot"])
+def test_rank_with_nothing_to_compute(cuda_device, op):
+    """More ranks than rows (elements): a rank with an empty shard still launches
+    its kernel and takes part in the exchange, and every rank gets the result."""
+    world = 4
+    if op == "dot":
+        nd = 3
+        x = synth.torch_uniform(synth.SEED_X, 0, 64, device=cuda_device)[:nd]
+        exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_DOT, 0, world, cuda_device)
+        parts = [partition_rows(nd, world, r) for r in range(world)]
+        assert any(b - a == 0 for a, b in parts)
+        ws, res = prealloc(world, "dot", 0, 64, (), cuda_device)
+        outs = run_ranks(world, lambda r: nvlink.lift_dot_allreduce(x[parts[r][0]:parts[r][1]],
+                                                                    x[parts[r][0]:parts[r][1]], exs[r],
+                                                                    out=res[r], workspace=ws[r]))
+        ref, mag = oracle.dot(x.cpu().numpy(), x.cpu().numpy())
+        for o in outs:
+            ok, margin = oracle.within_tol([o.item()], [ref], [mag])
+            assert ok, margin
+        return
+    m, n = 3, 512
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    B = synth.torch_matrix_rows(synth.SEED_B, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    full = lift.lift_gemv(A, x) if op == "gemv" else lift.lift_gesummv(1.5, A, 1.2, B, x)
+    exs = nvlink.ExchangeArea.simulated(nvlink.EXCH_GATHER, m, world, cuda_device)
+    parts = [partition_rows(m, world, r) for r in range(world)]
+    assert any(b - a == 0 for a, b in parts)
+    ws, res = prealloc(world, op, m, n, (m,), cuda_device)
+    for it in range(2):
+        outs = run_ranks(world, lambda r: nvlink.lift_gemv_allgather(
+            A[parts[r][0]:parts[r][1]], x, parts[r][0], m, exs[r], out=res[r], workspace=ws[r],
+            B=None if op == "gemv" else B[parts[r][0]:parts[r][1]], alpha=1.5, beta=1.2))
+        for r in range(world):
+            assert torch.equal(outs[r], full), (r, it)
