@@ -20,7 +20,13 @@
  *  - Ownership: the caller owns every buffer.  The library never allocates,
  *    frees, synchronises, or changes the current device.
  *  - Streams: `stream` is a cudaStream_t (NULL = legacy default stream).
- *    Work is enqueued asynchronously; calls are CUDA-graph capturable.
+ *    Work is enqueued asynchronously; calls are CUDA-graph capturable.  The
+ *    streaming kernels are launched with programmatic stream serialisation
+ *    (PDL): they may be scheduled while the previous kernel on the stream
+ *    drains, but each waits for it (griddepcontrol.wait) before touching
+ *    memory, so stream order is unchanged.  LIFT_PDL=0 in the environment
+ *    turns it off.  Waits inside a kernel (grid barriers) are bounded by
+ *    LIFT_SPIN_TIMEOUT_MS (default 20000) and trap when exceeded.
  *  - restrict: outputs must not overlap inputs or the workspace (Fig. 7
  *    declares `restrict` inputs, L948-950); overlap -> LIFT_ERR_ALIAS.
  *  - Errors: argument validation happens on the host BEFORE anything touches
