@@ -445,6 +445,9 @@ static int gather_common(int nmat, int64_t m, int64_t n, float alpha, const floa
     if (overlap(ry, rng(A, mat)) || overlap(ry, rng(x, (uint64_t)n * 4)) || (nmat == 2 && overlap(ry, rng(B, mat))) ||
         overlap(ry, rw))
         return LIFT_ERR_ALIAS;
+    // the ticket is written by the kernel: it must not live inside an input either
+    if (overlap(rw, rng(A, mat)) || overlap(rw, rng(x, (uint64_t)n * 4)) || (nmat == 2 && overlap(rw, rng(B, mat))))
+        return LIFT_ERR_ALIAS;
     if (m_total == 0) return LIFT_OK;
     DeviceInfo d;
     cudaError_t e = lift::device_info(&d);
@@ -490,10 +493,12 @@ int lift_atax_reduce(int64_t m, int64_t n, const float *A, const float *x, float
     if (st != LIFT_OK) return st;
     if (dst < -1 || dst >= world || blocks < 0) return LIFT_ERR_BAD_SIZE;
     if (!size_ok(m, n)) return LIFT_ERR_BAD_SIZE;
+    if (n > 0 && (y == nullptr || x == nullptr || (m > 0 && A == nullptr))) return LIFT_ERR_NULL_PTR;
+    if (n > 0 && (mis4(y) || mis4(x) || (m > 0 && mis4(A)))) return LIFT_ERR_MISALIGNED;
+    // 4-byte aligned but not 16: an unsupported shape for the fused kernel (as lift_atax FUSED)
     const bool aligned = ((reinterpret_cast<uintptr_t>(A) | reinterpret_cast<uintptr_t>(x) |
                            reinterpret_cast<uintptr_t>(y)) & 15) == 0;
     if (n > 0 && !lift::atax_fused_exchange_supported(m > 0 ? m : 1, n, aligned)) return LIFT_ERR_BAD_SIZE;
-    if (n > 0 && (y == nullptr || x == nullptr || (m > 0 && A == nullptr))) return LIFT_ERR_NULL_PTR;
     if (workspace == nullptr || workspace_bytes < lift_atax_workspace_bytes(m, n) ||
         (reinterpret_cast<uintptr_t>(workspace) & 15) != 0)
         return LIFT_ERR_WORKSPACE;

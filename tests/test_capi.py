@@ -236,6 +236,13 @@ def test_nvlink_validation():
     wsa = L.lift_atax_workspace_bytes(64, 512)
     assert L.lift_atax_reduce(64, 512, A_, X_, Y_, W_, wsa, peers, 0, 2, 2, 0, None) == SIZE      # dst >= world
     assert L.lift_atax_reduce(64, 510, A_, X_, Y_, W_, wsa, peers, 0, 2, 0, 0, None) == SIZE     # n % 4
+    assert L.lift_atax_reduce(64, 512, A_, X_ + 2, Y_, W_, wsa, peers, 0, 2, 0, 0, None) == MIS  # not 4-byte
+    assert L.lift_atax_reduce(64, 512, A_, X_ + 4, Y_, W_, wsa, peers, 0, 2, 0, 0, None) == SIZE  # not 16-byte
+    assert L.lift_atax_reduce(64, 512, A_, None, Y_, W_, wsa, peers, 0, 2, 0, 0, None) == NULL
+    assert L.lift_atax_reduce(64, 512, A_, X_, Y_, A_ + 256, wsa, peers, 0, 2, 0, 0, None) == ALIAS  # ws in A
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, Y_, A_ + 16, 256, peers, 0, 2, None) == ALIAS  # ticket in A
+    assert L.lift_gemv_allgather(10, 4, A_, X_, 0, 100, Y_, X_, 256, peers, 0, 2, None) == ALIAS       # ticket on x
+    assert L.lift_gesummv_allgather(10, 4, 1.0, A_, 1.0, B_, X_, 0, 10, Y_, B_, 256, peers, 0, 1, None) == ALIAS
 
 
 def test_host_entry_validation():
