@@ -52,6 +52,21 @@ def _same_device(*ts: torch.Tensor) -> torch.device:
     return d
 
 
+def _check_out(out: torch.Tensor, name: str, numel: int, device: torch.device) -> None:
+    """An output the kernels write: fp32, contiguous, on `device`, exactly `numel`
+    elements (the C ABI takes a bare pointer and cannot check its extent)."""
+    _check_tensor(out, name)
+    if out.device != device:
+        raise ValueError(f"{name} is on {out.device}, the inputs on {device}")
+    if out.numel() != numel:
+        raise ValueError(f"{name} has {out.numel()} elements, the result has {numel}")
+
+
+def _check_len(t: torch.Tensor, name: str, numel: int) -> None:
+    if t.numel() != numel:
+        raise ValueError(f"{name} has {t.numel()} elements, expected {numel}")
+
+
 _NULL_CTX = contextlib.nullcontext()
 
 
@@ -110,7 +125,7 @@ def lift_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None = None) 
         raise ValueError("x and y must have the same length")
     if out is None:
         out = torch.empty((), dtype=torch.float32, device=dev)
-    _check_tensor(out, "out")
+    _check_out(out, "out", 1, dev)
     L = lib()
     n = x.numel()
     nbytes = L.lift_dot_workspace_bytes(n)
@@ -131,6 +146,7 @@ def lift_gemv(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None)
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
+    _check_out(out, "out", m, dev)
     with _on(dev):
         check(lib().lift_gemv(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), _stream(dev)))
     return out
@@ -142,8 +158,10 @@ def lift_gemv_tuned(A, x, out=None, wpr=0, rg=0, blocks=0, xsmem=-1, lb=0):
     _check_tensor(x, "x", 1)
     dev = _same_device(A, x)
     m, n = A.shape
+    _check_len(x, "x", n)
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
+    _check_out(out, "out", m, dev)
     with _on(dev):
         check(lib().lift_gemv_tuned(m, n, A.data_ptr(), x.data_ptr(), out.data_ptr(), wpr, rg, blocks, xsmem, lb,
                                     _stream(dev)))
@@ -163,6 +181,7 @@ def lift_gesummv(alpha: float, A: torch.Tensor, beta: float, B: torch.Tensor, x:
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
+    _check_out(out, "out", m, dev)
     with _on(dev):
         check(lib().lift_gesummv(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
                                  out.data_ptr(), _stream(dev)))
@@ -175,8 +194,12 @@ def lift_gesummv_tuned(alpha, A, beta, B, x, out=None, wpr=0, rg=0, blocks=0, xs
     _check_tensor(x, "x", 1)
     dev = _same_device(A, B, x)
     m, n = A.shape
+    if tuple(B.shape) != (m, n):
+        raise ValueError("shape mismatch")
+    _check_len(x, "x", n)
     if out is None:
         out = torch.empty(m, dtype=torch.float32, device=dev)
+    _check_out(out, "out", m, dev)
     with _on(dev):
         check(lib().lift_gesummv_tuned(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
                                        out.data_ptr(), wpr, rg, blocks, xsmem, lb, _stream(dev)))
@@ -197,6 +220,7 @@ def lift_atax(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | None = None,
     if out is None:
         out = torch.empty(n, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
+    _check_out(out, "out", n, dev)
     L = lib()
     nbytes = L.lift_atax_workspace_bytes(m, n)
     with _on(dev):
@@ -218,6 +242,7 @@ def lift_atax_fused_tuned(A: torch.Tensor, x: torch.Tensor, out: torch.Tensor | 
     if out is None:
         out = torch.empty(n, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
+    _check_out(out, "out", n, dev)
     L = lib()
     nbytes = L.lift_atax_workspace_bytes(m, n)
     with _on(dev):
@@ -249,6 +274,7 @@ def lift_partial_dot(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None 
     if out is None:
         out = torch.empty(n // 128, dtype=torch.float32, device=dev)
     _check_tensor(out, "out", 1)
+    _check_out(out, "out", n // 128, dev)
     with _on(dev):
         check(lib().lift_partial_dot(n, x.data_ptr(), y.data_ptr(), out.data_ptr(), int(bool(contract)), _stream(dev)))
     return out
@@ -264,6 +290,7 @@ def lift_dot_listing1(x: torch.Tensor, y: torch.Tensor, out: torch.Tensor | None
         raise ValueError("x and y must have the same length")
     if out is None:
         out = torch.empty((), dtype=torch.float32, device=dev)
+    _check_out(out, "out", 1, dev)
     L = lib()
     n = x.numel()
     with _on(dev):
@@ -290,12 +317,18 @@ def lift_sgemv(alpha: float, A: torch.Tensor, x: torch.Tensor, beta: float = 0.0
         shape = tuple(A.shape) if lay == 0 else (A.shape[1], A.shape[0])
     m, n = shape
     ld = A.shape[1] if lda is None else lda
+    rows, cols = (m, n) if lay == 0 else (n, m)
+    if rows > 0 and cols > 0 and A.numel() < (rows - 1) * ld + cols:
+        raise ValueError(f"A holds {A.numel()} elements, a {rows} x {cols} matrix with lda {ld} needs "
+                         f"{(rows - 1) * ld + cols}")
     ylen = n if trans else m
     if y is None:
         if beta != 0.0:
             raise ValueError("beta != 0 needs y")
         y = torch.empty(ylen, dtype=torch.float32, device=dev)
     _check_tensor(y, "y", 1)
+    if y.device != dev:
+        raise ValueError(f"y is on {y.device}, A and x on {dev}")
     if y.numel() != ylen or x.numel() != (m if trans else n):
         raise ValueError("x / y length does not match op(A)")
     L = lib()
@@ -324,6 +357,10 @@ def lift_host_call(op: str, host: dict, dev: dict, alpha: float = 1.0, beta: flo
     for k, t in host.items():
         _check_host(t, k)
     device = next(iter(dev.values())).device
+    for k, t in host.items():  # the device buffers the copies land in: same extents
+        if k not in dev:
+            raise ValueError(f"no device buffer for {k}")
+        _check_out(dev[k], f"dev[{k!r}]", t.numel(), device)
     s = _stream(device)
     with torch.cuda.device(device):
         if op == "dot":

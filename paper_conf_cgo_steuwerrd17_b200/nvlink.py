@@ -19,7 +19,7 @@ from __future__ import annotations
 
 import torch
 
-from . import _check_tensor, _same_device, _stream, _workspace
+from . import _check_len, _check_out, _check_tensor, _same_device, _stream, _workspace
 from ._lib import check, lib
 
 EXCH_DOT, EXCH_GATHER, EXCH_REDUCE = 0, 1, 2
@@ -118,6 +118,14 @@ class ExchangeArea:
         return [cls(kind, length, areas[r], peers, r, world) for r in range(world)]
 
 
+def _check_area(ex: ExchangeArea, kind: int, length: int) -> None:
+    """The kernels size their stores by the call's shape: the area must have been
+    made for this kind and length (the device-side extent is not visible to them)."""
+    if ex.kind != kind or (kind != EXCH_DOT and ex.length != length):
+        raise ValueError(f"exchange area made for kind {ex.kind} length {ex.length}, the call needs kind {kind} "
+                         f"length {length}")
+
+
 def workspace_bytes(op: str, m: int = 0, n: int = 0) -> int:
     """Workspace bytes of one call (allocate zeroed, reuse across calls)."""
     L = lib()
@@ -140,9 +148,11 @@ def lift_dot_allreduce(x: torch.Tensor, y: torch.Tensor, ex: ExchangeArea, out: 
     _check_tensor(x, "x", 1)
     _check_tensor(y, "y", 1)
     dev = _same_device(x, y)
-    assert ex.kind == EXCH_DOT
+    _check_len(y, "y", x.numel())
+    _check_area(ex, EXCH_DOT, 0)
     if out is None:
         out = torch.empty((), dtype=torch.float32, device=dev)
+    _check_out(out, "out", 1, dev)
     L = lib()
     n = x.numel()
     with torch.cuda.device(dev):
@@ -161,10 +171,17 @@ def lift_gemv_allgather(A: torch.Tensor, x: torch.Tensor, row0: int, m_total: in
     _check_tensor(A, "A", 2)
     _check_tensor(x, "x", 1)
     dev = _same_device(A, x)
-    assert ex.kind == EXCH_GATHER and ex.length == m_total
+    _check_area(ex, EXCH_GATHER, m_total)
     m, n = A.shape
+    _check_len(x, "x", n)
+    if B is not None:
+        _check_tensor(B, "B", 2)
+        _same_device(A, B)
+        if tuple(B.shape) != (m, n):
+            raise ValueError(f"B has shape {tuple(B.shape)}, A {(m, n)}")
     if out is None:
         out = torch.empty(m_total, dtype=torch.float32, device=dev)
+    _check_out(out, "out", m_total, dev)
     L = lib()
     with torch.cuda.device(dev):
         ws = workspace if workspace is not None else _workspace(f"gather{ex.rank}", dev, 256, zero=True)
@@ -173,7 +190,6 @@ def lift_gemv_allgather(A: torch.Tensor, x: torch.Tensor, row0: int, m_total: in
                                        ws.numel(), ex.peers.data_ptr(), ex.rank, ex.world,
                                        _stream(dev))
         else:
-            _check_tensor(B, "B", 2)
             st = L.lift_gesummv_allgather(m, n, float(alpha), A.data_ptr(), float(beta), B.data_ptr(), x.data_ptr(),
                                           row0, m_total, out.data_ptr(), ws.data_ptr(), ws.numel(),
                                           ex.peers.data_ptr(), ex.rank, ex.world, _stream(dev))
@@ -188,9 +204,11 @@ def lift_atax_reduce(A: torch.Tensor, x: torch.Tensor, ex: ExchangeArea, dst: in
     _check_tensor(x, "x", 1)
     dev = _same_device(A, x)
     m, n = A.shape
-    assert ex.kind == EXCH_REDUCE and ex.length == n
+    _check_len(x, "x", n)
+    _check_area(ex, EXCH_REDUCE, n)
     if out is None:
         out = torch.empty(n, dtype=torch.float32, device=dev)
+    _check_out(out, "out", n, dev)
     L = lib()
     with torch.cuda.device(dev):
         ws = workspace if workspace is not None else _workspace(f"ataxr{ex.rank}", dev,

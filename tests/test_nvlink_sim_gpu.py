@@ -292,3 +292,36 @@ def test_rank_with_nothing_to_compute(cuda_device, op):
             B=None if op == "gemv" else B[parts[r][0]:parts[r][1]], alpha=1.5, beta=1.2))
         for r in range(world):
             assert torch.equal(outs[r], full), (r, it)
+
+
+def test_fused_binding_rejects_wrong_extents(cuda_device):
+    """The fused entry points' outputs, inputs and exchange areas are checked
+    against the call's shape before any launch (the kernels store by the call's
+    m / n into buffers whose extent they cannot see)."""
+    m, n = 64, 256
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    ex_dot = nvlink.ExchangeArea.simulated(nvlink.EXCH_DOT, 0, 1, cuda_device)[0]
+    ex_g = nvlink.ExchangeArea.simulated(nvlink.EXCH_GATHER, m, 1, cuda_device)[0]
+    ex_r = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n, 1, cuda_device)[0]
+    ex_r_small = nvlink.ExchangeArea.simulated(nvlink.EXCH_REDUCE, n // 2, 1, cuda_device)[0]
+    bad = [
+        lambda: nvlink.lift_dot_allreduce(x, x[:-1], ex_dot),
+        lambda: nvlink.lift_dot_allreduce(x, x, ex_dot, out=torch.empty(2, device=cuda_device)),
+        lambda: nvlink.lift_dot_allreduce(x, x, ex_g),
+        lambda: nvlink.lift_gemv_allgather(A, x, 0, m, ex_g, out=torch.empty(m - 1, device=cuda_device)),
+        lambda: nvlink.lift_gemv_allgather(A, x[:-4], 0, m, ex_g),
+        lambda: nvlink.lift_gemv_allgather(A, x, 0, m, ex_g, B=A[:-1]),
+        lambda: nvlink.lift_gemv_allgather(A, x, 0, 2 * m, ex_g),  # area made for m rows
+        lambda: nvlink.lift_atax_reduce(A, x, ex_r, out=torch.empty(n - 4, device=cuda_device)),
+        lambda: nvlink.lift_atax_reduce(A, x, ex_r_small),
+        lambda: nvlink.lift_atax_reduce(A, x, ex_g),
+    ]
+    for i, call in enumerate(bad):
+        with pytest.raises((ValueError, TypeError)):
+            call()
+            pytest.fail(f"case {i} accepted")
+    y = nvlink.lift_atax_reduce(A, x, ex_r)  # a valid call still runs
+    torch.cuda.synchronize()
+    ref, mag = oracle.atax(A.cpu().numpy(), x.cpu().numpy())
+    assert oracle.within_tol(y.cpu().numpy(), ref, mag)[0]

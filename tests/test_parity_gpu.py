@@ -676,3 +676,36 @@ def test_host_entry_points_match_device_path(cuda_device, pinned):
         lift.lift_host_call(op, h, d, alpha=1.5, beta=1.2)
         torch.cuda.synchronize()
         assert torch.equal(h["out"].reshape(-1), ref.cpu().reshape(-1)), op
+
+
+# ===================================================================== binding extents
+def test_binding_rejects_wrong_output_extents(cuda_device):
+    """The C ABI takes bare pointers and cannot see a buffer's extent: the binding
+    rejects an output (or tuned input) of the wrong length or device before any
+    launch, so a short tensor is never written past its end."""
+    m, n = 64, 256
+    A = synth.torch_matrix_rows(synth.SEED_A, n, 0, m, device=cuda_device)
+    x = synth.torch_uniform(synth.SEED_X, 0, n, device=cuda_device)
+    short_m, short_n = torch.empty(m - 1, device=cuda_device), torch.empty(n - 4, device=cuda_device)
+    bad = [
+        lambda: lift.lift_gemv(A, x, out=short_m),
+        lambda: lift.lift_gemv_tuned(A, x, out=short_m),
+        lambda: lift.lift_gemv_tuned(A, x[:-4]),
+        lambda: lift.lift_gesummv(1.0, A, 1.0, A, x, out=short_m),
+        lambda: lift.lift_gesummv_tuned(1.0, A, 1.0, A[:-1], x),
+        lambda: lift.lift_atax(A, x, out=short_n),
+        lambda: lift.lift_atax_fused_tuned(A, x, out=short_n),
+        lambda: lift.lift_dot(x, x, out=torch.empty(0, device=cuda_device)),
+        lambda: lift.lift_dot_listing1(x, x, out=torch.empty(2, device=cuda_device)),
+        lambda: lift.lift_partial_dot(x, x, out=torch.empty(1, device=cuda_device)),
+        lambda: lift.lift_gemv(A, x, out=torch.empty(m)),  # host tensor
+        lambda: lift.lift_sgemv(1.0, A[:10], x, shape=(m, n)),  # A shorter than the matrix
+        lambda: lift.lift_host_call("gemv", dict(A=A.cpu(), x=x.cpu(), out=torch.empty(m)),
+                                    dict(A=A, x=x, out=short_m)),
+    ]
+    for i, call in enumerate(bad):
+        with pytest.raises((ValueError, TypeError)):
+            call()
+            pytest.fail(f"case {i} accepted")
+    torch.cuda.synchronize()
+    assert torch.equal(lift.lift_gemv_tuned(A, x), lift.lift_gemv(A, x))  # the checks pass valid calls
