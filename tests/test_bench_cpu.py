@@ -124,3 +124,26 @@ def test_table1_calls_bind_their_own_operands(monkeypatch):
                 assert s[1] == (shp["m"], shp["n"]) and s[3] == shp["m"]
             else:
                 assert s[1] == (shp["m"], shp["n"]) and s[3] == shp["n"]
+
+
+def test_clock_rejection_rule():
+    """The contract's rejection rule on the NVML samples of a timed region:
+    thermal / hardware slowdowns reject, sw_power_cap is kept (and noted), and
+    clocks far below max with no reason (a leftover clock lock) reject."""
+    def sampler(samples, reasons, max_mhz=1965):
+        s = bench.ClockSampler.__new__(bench.ClockSampler)
+        s.ok, s.samples, s.reasons, s.max_mhz = True, samples, reasons, max_mhz
+        return s
+
+    assert not sampler([1950, 1965], 0).rejectable()
+    assert not sampler([1800, 1810], 0x4).rejectable()          # sw_power_cap: kept
+    assert "sw_power_cap" in sampler([1800], 0x4).summary()["reasons"]
+    assert sampler([1900], 0x8).rejectable()                    # hw_slowdown
+    assert sampler([1900], 0x20).rejectable()                   # sw_thermal_slowdown
+    assert sampler([1900], 0x40 | 0x4).rejectable()             # hw_thermal_slowdown
+    assert sampler([1000, 1005], 0).rejectable()                # stuck low, no reason
+    assert not sampler([1000, 1005], 0x4).rejectable()          # low but power-capped: noted, kept
+    assert sampler([1000], 0x1).rejectable()                    # gpu_idle is not a reason: low clocks reject
+    s = bench.ClockSampler.__new__(bench.ClockSampler)
+    s.ok, s.samples, s.reasons, s.max_mhz = False, [], 0, None
+    assert not s.rejectable()                                   # NVML unavailable: nothing to judge
