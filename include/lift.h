@@ -21,7 +21,8 @@
  *    frees, synchronises, or changes the current device.
  *  - Streams: `stream` is a cudaStream_t (NULL = legacy default stream).
  *    Work is enqueued asynchronously; calls are CUDA-graph capturable.  The
- *    streaming kernels are launched with programmatic stream serialisation
+ *    kernels (all but the fused collectives of lift_nvlink.h) are launched
+ *    with programmatic stream serialisation
  *    (PDL): they may be scheduled while the previous kernel on the stream
  *    drains, but each waits for it (griddepcontrol.wait) before touching
  *    memory, so stream order is unchanged.  LIFT_PDL=0 in the environment

@@ -606,6 +606,8 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         fence_mbar_init();
     }
     __syncthreads();
+    pdl_wait();                        // no global access before the previous kernel is complete
+    if (ex.world == 0) pdl_release();  // (a no-op unless launched with the PDL attribute)
     if (tid == 0)  // prologue: fill the ring
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
     // fused (all-)reduce: this call's epoch (its parity buffer is free: the previous
@@ -792,7 +794,7 @@ static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m,
     auto k = k_atax_fused<QC, CR>;
     cudaError_t e = ensure_smem(k, d.device, p.smem);
     if (e != cudaSuccess) return e;
-    cudaLaunchAttribute attr[1];
+    cudaLaunchAttribute attr[2];
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3((unsigned)blocks);
     cfg.blockDim = dim3(kFusedThreads);
@@ -804,6 +806,15 @@ static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m,
         attr[0].id = cudaLaunchAttributeCooperative;
         attr[0].val.cooperative = 1;
         cfg.numAttrs = 1;
+    }
+    // programmatic dependent launch (common.cuh): the launch and this kernel's barrier
+    // setup overlap the previous kernel's tail (-0.4..0.6 us per call,
+    // profiles/r02_atax_pdl_ab.txt); the kernel reads no global memory before its
+    // griddepcontrol.wait.  Not for the fused collectives (see launch_pdl).
+    if (ex.world == 0 && pdl_enabled()) {
+        attr[cfg.numAttrs].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+        attr[cfg.numAttrs].val.programmaticStreamSerializationAllowed = 1;
+        ++cfg.numAttrs;
     }
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, ex, dst, p.cyc,
                               rows_are_lines(P, n));
@@ -856,6 +867,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         fence_mbar_init();
     }
     cluster_sync();  // every block's barriers initialised before anyone pushes into it
+    pdl_wait_and_release();  // no global access before the previous kernel is complete
     if (tid == 0)
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
 
@@ -961,7 +973,7 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
         }
     }
     if (e != cudaSuccess) return e;
-    cudaLaunchAttribute attr[1];
+    cudaLaunchAttribute attr[2];
     attr[0].id = cudaLaunchAttributeClusterDimension;
     attr[0].val.clusterDim.x = (unsigned)C;
     attr[0].val.clusterDim.y = 1;
@@ -1018,13 +1030,21 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
         const char *v = getenv("LIFT_WIDE_COOPERATIVE");
         return !(v && v[0] == '0');
     }();
-    cudaLaunchAttribute attr2[2] = {attr[0], {}};
+    cudaLaunchAttribute attr2[3] = {attr[0], {}, {}};
     attr2[1].id = cudaLaunchAttributeCooperative;
     attr2[1].val.cooperative = 1;
+    int na2 = 2;
+    if (pdl_enabled()) {  // as the single-block kernel (run_fused)
+        attr[1].id = attr2[2].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+        attr[1].val.programmaticStreamSerializationAllowed = attr2[2].val.programmaticStreamSerializationAllowed = 1;
+        cfg.numAttrs = 2;
+        na2 = 3;
+    }
     const int dev = d.device >= 0 && d.device < 64 ? d.device : 0;
     if (coop_env && coop_ok[dev] >= 0) {
+        const int na1 = cfg.numAttrs;
         cfg.attrs = attr2;
-        cfg.numAttrs = 2;
+        cfg.numAttrs = na2;
         cudaError_t e2 = cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
         if (e2 == cudaSuccess) {
             coop_ok[dev] = 1;
@@ -1034,7 +1054,7 @@ static cudaError_t run_wide(const DeviceInfo &d, const WidePlan &p, int64_t m, i
         (void)cudaGetLastError();  // refused: remember, launch plainly
         coop_ok[dev] = -1;
         cfg.attrs = attr;
-        cfg.numAttrs = 1;
+        cfg.numAttrs = na1;
     }
     return cudaLaunchKernelEx(&cfg, k, m, n, p.nst, (int)p.hdr, A, x, P, y, gbar, rows_are_lines(P, n));
 }
