@@ -43,6 +43,22 @@ namespace lift {
 
 constexpr int kMaxSplits = 256;  // partial-row capacity of the workspace
 
+// Phase timestamps of the single-block fused kernel, compiled in only for the
+// timeline probe (tools/atax_trace.py builds a separate library with
+// -DLIFT_TRACE); the product library has none of it.
+#ifdef LIFT_TRACE
+constexpr int kTraceSlots = 16;
+__device__ unsigned long long g_trace[kMaxSplits * kTraceSlots];
+#define LIFT_STAMP(k)                                                                          \
+    do {                                                                                       \
+        if (threadIdx.x == 0) g_trace[blockIdx.x * kTraceSlots + (k)] = globaltimer_ns();      \
+    } while (0)
+#else
+#define LIFT_STAMP(k) \
+    do {              \
+    } while (0)
+#endif
+
 static inline size_t align256(size_t b) { return (b + 255) / 256 * 256; }
 
 // workspace: [0, 256) grid-barrier counters (zero before first use, left zero),
@@ -449,6 +465,27 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
         }
         part[sp * CW + col] = acc;
         __syncthreads();  // every load of this pass has been consumed
+#ifdef LIFT_TRACE
+        if (cb == c0) LIFT_STAMP(7);
+#ifdef LIFT_TRACE_REPEAT  // the same loads once more (now certainly L2 hits): their latency alone
+        if (cb == c0) {
+            float4 acc2 = zero4();
+            if (c < c1)
+                for (int s = s0; s < s1; s += IF) {
+                    float4 v[IF];
+#pragma unroll
+                    for (int u = 0; u < IF; ++u)
+                        if (s + u < s1) v[u] = __ldcg(P4 + (int64_t)(s + u) * nv + c);
+#pragma unroll
+                    for (int u = 0; u < IF; ++u)
+                        if (s + u < s1) acc2.x += v[u].x + v[u].y + v[u].z + v[u].w;
+                }
+            if (acc2.x == 12345.f) part[0] = acc2;  // keep the loads
+            __syncthreads();
+            LIFT_STAMP(8);
+        }
+#endif
+#endif
         if (discard) {    // its lines (2 per row) of every partial row are dead now
             const int64_t e = cb + CW < c1 ? cb + CW : c1;
             const int nl = (int)((e - cb + 7) / 8);
@@ -608,6 +645,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     __syncthreads();
     pdl_wait();                        // no global access before the previous kernel is complete
     if (ex.world == 0) pdl_release();  // (a no-op unless launched with the PDL attribute)
+    LIFT_STAMP(0);
     if (tid == 0)  // prologue: fill the ring
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
     // fused (all-)reduce: this call's epoch (its parity buffer is free: the previous
@@ -654,6 +692,10 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         float *rb = red + buf * CR * kFusedWarps;
         if (rows > 0) {
             mbar_wait_parity(full + slot, phase);
+#ifdef LIFT_TRACE
+            if (k == 0) LIFT_STAMP(1);
+            if (k == nstg / 2) LIFT_STAMP(2);
+#endif
             const float4 *S4 = reinterpret_cast<const float4 *>(stage0 + (size_t)slot * stage_floats);
 #pragma unroll
             for (int i = 0; i < CR; ++i) {
@@ -713,6 +755,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         if (step(ra, rb2)) break;
         if (step(rb2, ra)) break;
     }
+    LIFT_STAMP(3);
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
 #pragma unroll
     for (int q = 0; q < QC; ++q) {
@@ -722,7 +765,9 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
 
     // ---- second stage in the same launch: grid barrier, then every block sums
     // a slice of the columns over all G partial rows in a fixed order ----
+    LIFT_STAMP(4);
     grid_barrier(gbar);
+    LIFT_STAMP(5);
     // every block sums its own slice of columns (the drained ring holds the split sums);
     // when the partial rows are whole 128-byte lines the slices are too, and each block
     // discards the lines it has read (no DRAM write-back of dead partials)
@@ -731,6 +776,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     int64_t c0 = unit * (nu * blockIdx.x / gridDim.x), c1 = unit * (nu * (blockIdx.x + 1) / gridDim.x);
     if (c1 > nv) c1 = nv;
     colsum_slice<8>((int)gridDim.x, nv, P, y, c0, c1, reinterpret_cast<float4 *>(stage0), lines);
+    LIFT_STAMP(6);
     if (ex.world == 0) {
         grid_depart(gbar);
         return;
@@ -1082,6 +1128,12 @@ cudaError_t atax_fused_grid(const DeviceInfo &d, int64_t m, int64_t n, int *bloc
     if (w.clu == 8) return run_wide<8>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
     return run_wide<16>(d, w, m, n, nullptr, nullptr, nullptr, nullptr, nullptr, 0, blocks);
 }
+
+#ifdef LIFT_TRACE
+extern "C" __attribute__((visibility("default"))) int lift_trace_copy(void *host, size_t bytes) {
+    return (int)cudaMemcpyFromSymbol(host, g_trace, bytes < sizeof(g_trace) ? bytes : sizeof(g_trace));
+}
+#endif
 
 cudaError_t preload_atax() {  // see preload_dot (dot.cu)
     cudaFuncAttributes a;
