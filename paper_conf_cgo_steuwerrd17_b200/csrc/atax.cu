@@ -632,10 +632,13 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         const int64_t a = stage_row(j);
         return (int)((r1 - a) < CR ? (r1 - a) : CR);
     };
+    // A is read once: its lines go first when L2 needs room (-0.15..0.3 us per call,
+    // profiles/r02_atax_evict_first_ab.txt)
+    const uint64_t pol = l2_policy_evict_first();
     auto issue_stage = [&](int64_t j, int slot) {
         const uint32_t bytes = (uint32_t)((int64_t)stage_rows(j) * n * 4);
         mbar_arrive_expect_tx(full + slot, bytes);
-        bulk_g2s(stage0 + (size_t)slot * stage_floats, A + stage_row(j) * n, bytes, full + slot);
+        bulk_g2s_hint(stage0 + (size_t)slot * stage_floats, A + stage_row(j) * n, bytes, full + slot, pol);
     };
 
     if (tid == 0) {
@@ -902,9 +905,10 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     const int64_t nstages = kc < m ? (m - kc + K - 1) / K : 0;  // rows kc, kc+K, ...
     constexpr int SB = C * kFusedWarps;
     constexpr uint32_t kStepBytes = SB * 4;
+    const uint64_t pol = l2_policy_evict_first();  // as k_atax_fused
     auto issue_stage = [&](int64_t j, int slot) {
         mbar_arrive_expect_tx(full + slot, (uint32_t)(nc * 4));
-        bulk_g2s(stage0 + (size_t)slot * nc, A + (j * K + kc) * n + col0, (uint32_t)(nc * 4), full + slot);
+        bulk_g2s_hint(stage0 + (size_t)slot * nc, A + (j * K + kc) * n + col0, (uint32_t)(nc * 4), full + slot, pol);
     };
     if (tid == 0) {
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);

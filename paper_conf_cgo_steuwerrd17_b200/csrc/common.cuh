@@ -319,6 +319,23 @@ __device__ __forceinline__ void bulk_g2s(void *dst_smem, const void *src_gmem, u
         : "memory");
 }
 
+// The same with an L2 eviction-priority hint: `policy` from l2_policy_evict_first()
+// marks the streamed lines as the first to go, so a single-use stream does not
+// push the kernel's own instructions and small reused data out of L2.
+__device__ __forceinline__ uint64_t l2_policy_evict_first() {
+    uint64_t pol;
+    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
+    return pol;
+}
+__device__ __forceinline__ void bulk_g2s_hint(void *dst_smem, const void *src_gmem, uint32_t bytes, uint64_t *bar,
+                                              uint64_t policy) {
+    asm volatile(
+        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], "
+        "%4;" ::"r"(smem_u32(dst_smem)),
+        "l"(src_gmem), "r"(bytes), "r"(smem_u32(bar)), "l"(policy)
+        : "memory");
+}
+
 // Prefetch `bytes` (multiple of 16) of gmem into L2 with the bulk-copy engine
 // (no smem, no completion tracking).
 __device__ __forceinline__ void bulk_prefetch_l2(const void *src_gmem, uint32_t bytes) {
