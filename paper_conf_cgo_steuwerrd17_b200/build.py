@@ -20,7 +20,8 @@ SO = os.path.join(PKG, "liblift.so")
 UNITS = ["capi.cu", "dot.cu", "gemv.cu", "atax.cu", "listing1.cu"]
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 NVCC_FLAGS = ARCH + ["-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC,-fvisibility=hidden",
-                     "-I", INCLUDE, "-I", CSRC, "--expt-relaxed-constexpr"]
+                     "-I", INCLUDE, "-I", CSRC, "--expt-relaxed-constexpr"] + \
+    os.environ.get("LIFT_NVCC_EXTRA", "").split()  # experiment switches (-D...) for A/B builds
 
 
 def _nvcc() -> str:

@@ -9,7 +9,8 @@ import sys
 
 import torch
 
-ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+# LIFT_ROOT: the package root to time (tools/ab_tree.sh points it at an older tree)
+ROOT = os.environ.get("LIFT_ROOT") or os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 sys.path.insert(0, os.path.join(ROOT, "tools"))
 import bench  # noqa: E402
