@@ -646,8 +646,12 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         fence_mbar_init();
     }
     __syncthreads();
-    pdl_wait();                        // no global access before the previous kernel is complete
-    if (ex.world == 0) pdl_release();  // (a no-op unless launched with the PDL attribute)
+    // no global access before the previous kernel is complete (a no-op unless launched
+    // with the PDL attribute).  No launch_dependents: the next kernel launches at this
+    // one's completion — triggered any earlier, even after the main loop, the 8 GiB-class
+    // GEMV that follows in the bench step ran 17-20 us slower
+    // (profiles/r02_atax_pdl_trigger_ab.txt)
+    pdl_wait();
     LIFT_STAMP(0);
     if (tid == 0)  // prologue: fill the ring
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
@@ -857,9 +861,9 @@ static cudaError_t run_fused(const DeviceInfo &d, const FusedPlan &p, int64_t m,
         cfg.numAttrs = 1;
     }
     // programmatic dependent launch (common.cuh): the launch and this kernel's barrier
-    // setup overlap the previous kernel's tail (-0.4..0.6 us per call,
-    // profiles/r02_atax_pdl_ab.txt); the kernel reads no global memory before its
-    // griddepcontrol.wait.  Not for the fused collectives (see launch_pdl).
+    // setup overlap the previous kernel's tail (profiles/r02_atax_pdl_ab.txt); the
+    // kernel reads no global memory before its griddepcontrol.wait and never triggers
+    // its own dependents early.  Not for the fused collectives (see launch_pdl).
     if (ex.world == 0 && pdl_enabled()) {
         attr[cfg.numAttrs].id = cudaLaunchAttributeProgrammaticStreamSerialization;
         attr[cfg.numAttrs].val.programmaticStreamSerializationAllowed = 1;
@@ -917,7 +921,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         fence_mbar_init();
     }
     cluster_sync();  // every block's barriers initialised before anyone pushes into it
-    pdl_wait_and_release();  // no global access before the previous kernel is complete
+    pdl_wait();  // no global access before the previous kernel is complete (no early trigger: k_atax_fused)
     if (tid == 0)
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
 

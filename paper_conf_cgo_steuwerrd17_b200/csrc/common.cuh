@@ -134,8 +134,8 @@ static inline cudaError_t ensure_smem(K kern, int dev, size_t smem) {
 // starts with griddepcontrol.wait (before ANY global memory access: the
 // previous kernel may produce its inputs or read its outputs) and then lets
 // its own dependent launch.  The cooperative fused ATAX kernels take the same
-// attribute beside their cooperative / cluster ones (atax.cu); the fused
-// collectives do not (launch_pdl's `allow`).
+// attribute beside their cooperative / cluster ones but never trigger early
+// (atax.cu); the fused collectives do not take it (launch_pdl's `allow`).
 // LIFT_PDL=0 turns it off (A/B).
 // ---------------------------------------------------------------------------
 __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
