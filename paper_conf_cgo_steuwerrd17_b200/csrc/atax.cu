@@ -644,6 +644,11 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     if (tid == 0) {
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         fence_mbar_init();
+#if LIFT_PDL_PREFETCH
+        // the ring's first stages into L2 while the previous kernel drains (common.cuh)
+        for (int i = 0; i < nst && i < nstages; ++i)
+            bulk_prefetch_l2(A + stage_row(i) * n, (uint32_t)((int64_t)stage_rows(i) * n * 4));
+#endif
     }
     __syncthreads();
     // no global access before the previous kernel is complete (a no-op unless launched

@@ -139,6 +139,15 @@ static inline cudaError_t ensure_smem(K kern, int dev, size_t smem) {
 // LIFT_PDL=0 turns it off (A/B).
 // ---------------------------------------------------------------------------
 __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+// Before its griddepcontrol.wait a dependent block may already pull the first
+// bytes of its READ-ONLY stream into L2 (cp.async.bulk.prefetch.L2, issued
+// while the previous kernel drains).  A prefetch returns nothing to the
+// program and L2 is the device's point of coherence, so even a range the
+// previous kernel is still writing cannot be read stale: only the loads after
+// pdl_wait() deliver data.  -DLIFT_PDL_PREFETCH=0 compiles it out (A/B).
+#ifndef LIFT_PDL_PREFETCH
+#define LIFT_PDL_PREFETCH 1
+#endif
 __device__ __forceinline__ void pdl_release() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
 __device__ __forceinline__ void pdl_wait_and_release() {
     pdl_wait();

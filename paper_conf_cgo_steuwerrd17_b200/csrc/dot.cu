@@ -37,9 +37,19 @@ __device__ __forceinline__ float block_sum(float v, float *red) {
 template <int TPB, int U, bool VEC>
 __global__ void __launch_bounds__(TPB) k_dot(int64_t n, const float *__restrict__ x, const float *__restrict__ y,
                                              float *__restrict__ result, float *__restrict__ partials,
-                                             unsigned int *__restrict__ ticket, Exch ex) {
+                                             unsigned int *__restrict__ ticket, Exch ex, int pf_blocks) {
     __shared__ float red[TPB / kWarp];
     __shared__ bool am_last;
+    if constexpr (VEC && LIFT_PDL_PREFETCH) {
+        // the first resident wave: this block's first U chunks of x and y into L2
+        // while the previous kernel drains (common.cuh); lane u of warp 0 takes chunk u
+        const int64_t n4 = n >> 2, i0 = (int64_t)blockIdx.x * TPB + (int64_t)threadIdx.x * gridDim.x * TPB;
+        if ((int)blockIdx.x < pf_blocks && threadIdx.x < U && i0 < n4) {
+            const uint32_t bytes = (uint32_t)((n4 - i0 < TPB ? n4 - i0 : TPB) * 16);
+            bulk_prefetch_l2(x + 4 * i0, bytes);
+            bulk_prefetch_l2(y + 4 * i0, bytes);
+        }
+    }
     pdl_wait();
     if (ex.world == 0) pdl_release();  // a fused collective lets nothing start early beside it
     const int64_t stride = (int64_t)gridDim.x * TPB;
@@ -174,8 +184,9 @@ cudaError_t launch_dot(const DeviceInfo &d, int64_t n, const float *x, const flo
     int64_t cap = (int64_t)d.sms * per_sm * (units < kOneWaveUnits ? 1 : kWaves);
     if (cap > kDotMaxBlocks) cap = kDotMaxBlocks;
     int blocks = (int)(want < 1 ? 1 : (want > cap ? cap : want));
-    if (vec) return launch_pdl(ex.world == 0, k_dot<TPB, U, true>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex);
-    return launch_pdl(ex.world == 0, k_dot<TPB, U, false>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex);
+    const int pf_blocks = d.sms * per_sm;  // blocks of the first resident wave
+    if (vec) return launch_pdl(ex.world == 0, k_dot<TPB, U, true>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex, pf_blocks);
+    return launch_pdl(ex.world == 0, k_dot<TPB, U, false>, dim3(blocks), dim3(TPB), 0, s, n, x, y, result, partials, ticket, ex, pf_blocks);
 }
 
 // Load every kernel of this unit now (CUDA's lazy loading would otherwise load a

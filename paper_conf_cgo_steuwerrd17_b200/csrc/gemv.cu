@@ -68,7 +68,7 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
                                                         const float *__restrict__ A, const float *__restrict__ B,
                                                         const float *__restrict__ x, float *__restrict__ y,
                                                         float alpha, float beta, int epi, Exch ex, int64_t row0,
-                                                        int64_t m_total, unsigned int *ticket) {
+                                                        int64_t m_total, unsigned int *ticket, int pf_blocks) {
     using V = Vec<VEC>;
     using T = typename V::T;
     constexpr int KQ = kSlices / WPR;                                 // slices per warp
@@ -78,11 +78,23 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     float *red = reinterpret_cast<float *>(smem + 16);
     float *xs = reinterpret_cast<float *>(smem + gemv_x_offset<NMAT, RG>());
 
-    pdl_wait();
-    if (ex.world == 0) pdl_release();  // a fused collective lets nothing start early beside it
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int g = warp / WPR;   // row group inside the block
     const int wr = warp % WPR;  // warp rank inside the row group
+    if constexpr (VEC == 4 && LIFT_PDL_PREFETCH) {
+        // the first resident wave's first rows (A and B are never written by this
+        // kernel), up to the 16 KiB of a row the first load batches cover, into L2
+        // while the previous kernel drains (common.cuh).  Later waves start beside
+        // running blocks, not after a predecessor: nothing to hide there.
+        const int64_t r = (int64_t)blockIdx.x * RG + g;
+        if ((int)blockIdx.x < pf_blocks && wr == 0 && lane == 0 && r < m && n > 0) {
+            const uint32_t bytes = (uint32_t)(n * 4 < 16384 ? n * 4 : 16384);
+            bulk_prefetch_l2(A + r * lda, bytes);
+            if constexpr (NMAT == 2) bulk_prefetch_l2(B + r * lda, bytes);
+        }
+    }
+    pdl_wait();
+    if (ex.world == 0) pdl_release();  // a fused collective lets nothing start early beside it
     const int64_t nv = n / VEC;
     const int64_t kcount = (nv + kVLanes - 1) / kVLanes;  // k-steps per row
     const int64_t kfull = nv / kVLanes;                   // k-steps whose every vector is in the row
@@ -301,8 +313,10 @@ static cudaError_t run_gemv(const DeviceInfo &d, const GemvArgs &a, int blocks, 
     if (groups >= 32 * cap) cap *= 4;
     int64_t g = blocks > 0 ? blocks : (groups < cap ? groups : cap);
     if (g < 1) g = 1;
+    const int64_t wave = (int64_t)per_sm * d.sms;  // blocks of the first resident wave
+    const int pf_blocks = (int)(g < wave ? g : wave);
     return launch_pdl(a.ex.world == 0, kern, dim3((unsigned)g), dim3(threads), smem, s, a.m, a.n, a.lda, a.A, a.B, a.x, a.y, a.alpha,
-                      a.beta, a.epi, a.ex, a.row0, a.m_total, a.ticket);
+                      a.beta, a.epi, a.ex, a.row0, a.m_total, a.ticket, pf_blocks);
 }
 
 template <int NMAT, int VEC, bool XSMEM>
