@@ -157,10 +157,17 @@ __global__ void __launch_bounds__(TPB) k_atax_cols(int64_t m, int64_t n, int64_t
                                                    const float *__restrict__ A, const float *__restrict__ t,
                                                    float *__restrict__ P) {
     using V = typename std::conditional<VEC == 4, float4, float>::type;
-    pdl_wait_and_release();
     const int s = blockIdx.y;
     const int64_t r0 = m * s / S, r1 = m * (s + 1) / S;
     const int64_t nv = n / VEC;
+    if constexpr (VEC == 4 && LIFT_PDL_PREFETCH) {
+        // this block's first 2*UR row segments into L2 while the previous kernel
+        // (pass 1, which writes t, never A) drains (common.cuh); one wave of blocks
+        const int64_t cb = (int64_t)blockIdx.x * TPB;
+        if (threadIdx.x < 2 * UR && r0 + threadIdx.x < r1 && cb < nv)
+            bulk_prefetch_l2(A + (r0 + threadIdx.x) * lda + 4 * cb, (uint32_t)((nv - cb < TPB ? nv - cb : TPB) * 16));
+    }
+    pdl_wait_and_release();
     const int64_t c = (int64_t)blockIdx.x * TPB + threadIdx.x;
     if (c >= nv) return;
     const int64_t ldv = lda / VEC;  // row stride in vectors
@@ -924,6 +931,10 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         for (int i = 0; i < R; ++i) mbar_init(sfull + i, 1);
         for (int i = 0; i < kFusedMaxStages; ++i) used[i] = 0u;
         fence_mbar_init();
+#if LIFT_PDL_PREFETCH
+        // the ring's first row slices into L2 while the previous kernel drains (common.cuh)
+        for (int i = 0; i < nst && i < nstages; ++i) bulk_prefetch_l2(A + (i * K + kc) * n + col0, (uint32_t)(nc * 4));
+#endif
     }
     cluster_sync();  // every block's barriers initialised before anyone pushes into it
     pdl_wait();  // no global access before the previous kernel is complete (no early trigger: k_atax_fused)
