@@ -31,7 +31,7 @@ def mats(cuda_device):
 
 
 def chain(A, x, outs):
-    """One pass: 9 ops (13 kernels), each consuming the previous results."""
+    """One pass: 13 ops (17 kernels), each consuming the previous results."""
     A1, A2, A3, A4 = A
     lift.lift_gemv(A1, x, out=outs["y1"])
     lift.lift_atax(A2, outs["y1"], out=outs["y2"], algo="fused")
@@ -43,11 +43,21 @@ def chain(A, x, outs):
     lift.lift_partial_dot(outs["y5"], outs["y3"], out=outs["z7"])
     lift.lift_gemv(A3, outs["y5"], out=outs["y8"])
     lift.lift_dot_listing1(outs["y8"], outs["y8"], out=outs["s9"])
+    # a MATRIX produced by the kernel right before: the dependent GEMV / fused ATAX
+    # blocks prefetch their first rows into L2 before griddepcontrol.wait, while the
+    # producer (which lets its dependents launch at its start) may still be writing
+    # them; only the loads after the wait may deliver data (common.cuh)
+    lift.lift_gemv(A3, outs["y8"], out=outs["y10"])
+    lift.lift_gemv(outs["y10"].view(16, 256), outs["y1"][:256], out=outs["y11"])
+    lift.lift_gemv(A4, outs["y10"], out=outs["y12"])
+    lift.lift_atax(outs["y12"].view(16, 256), outs["y1"][:256], out=outs["y13"], algo="fused")
 
 
 def fresh_outputs(device):
     nan = float("nan")
-    o = {k: torch.full((N,), nan, device=device) for k in ("y1", "y2", "y3", "y4", "y5", "y8")}
+    o = {k: torch.full((N,), nan, device=device) for k in ("y1", "y2", "y3", "y4", "y5", "y8", "y10", "y12")}
+    o["y11"] = torch.full((16,), nan, device=device)
+    o["y13"] = torch.full((256,), nan, device=device)
     o["s6"] = torch.full((), nan, device=device)
     o["s9"] = torch.full((), nan, device=device)
     o["z7"] = torch.full((N // 128,), nan, device=device)
@@ -75,6 +85,10 @@ def check_chain(A, x, outs):
     ok("dot", h["s6"], oracle.dot(h["y5"], h["y1"]))
     ok("partial dot", h["z7"], oracle.partial_dot(h["y5"], h["y3"]))
     ok("gemv 2", h["y8"], oracle.gemv(A3, h["y5"]))
+    ok("gemv 3", h["y10"], oracle.gemv(A3, h["y8"]))
+    ok("gemv of a produced matrix", h["y11"], oracle.gemv(h["y10"].reshape(16, 256), h["y1"][:256]))
+    ok("gemv 4", h["y12"], oracle.gemv(A4, h["y10"]))
+    ok("atax of a produced matrix", h["y13"], oracle.atax(h["y12"].reshape(16, 256), h["y1"][:256]))
     assert np.float32(h["s9"]).view(np.uint32) == np.float32(oracle.dot_listing1_f32(h["y8"], h["y8"])).view(
         np.uint32), "listing-1 dot differs from the paper-order emulation"
 
