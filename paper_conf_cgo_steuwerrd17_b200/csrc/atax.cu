@@ -652,8 +652,13 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         fence_mbar_init();
 #if LIFT_PDL_PREFETCH
-        // the ring's first stages into L2 while the previous kernel drains (common.cuh)
-        for (int i = 0; i < nst && i < nstages; ++i)
+        // the ring's first stages into L2 while the previous kernel drains (common.cuh);
+        // twice or four times the ring is slower (4096^2 15.5 -> 17.4 / 19.1 us,
+        // profiles/r02_pdl_prefetch_depth_ab.txt)
+#ifndef LIFT_ATAX_PF_MULT
+#define LIFT_ATAX_PF_MULT 1
+#endif
+        for (int i = 0; i < LIFT_ATAX_PF_MULT * nst && i < nstages; ++i)
             bulk_prefetch_l2(A + stage_row(i) * n, (uint32_t)((int64_t)stage_rows(i) * n * 4));
 #endif
     }

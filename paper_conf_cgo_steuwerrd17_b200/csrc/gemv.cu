@@ -82,15 +82,26 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     const int g = warp / WPR;   // row group inside the block
     const int wr = warp % WPR;  // warp rank inside the row group
     if constexpr (VEC == 4 && LIFT_PDL_PREFETCH) {
-        // the first resident wave's first rows (A and B are never written by this
-        // kernel), up to the 16 KiB of a row the first load batches cover, into L2
-        // while the previous kernel drains (common.cuh).  Later waves start beside
-        // running blocks, not after a predecessor: nothing to hide there.
-        const int64_t r = (int64_t)blockIdx.x * RG + g;
-        if ((int)blockIdx.x < pf_blocks && wr == 0 && lane == 0 && r < m && n > 0) {
-            const uint32_t bytes = (uint32_t)(n * 4 < 16384 ? n * 4 : 16384);
-            bulk_prefetch_l2(A + r * lda, bytes);
-            if constexpr (NMAT == 2) bulk_prefetch_l2(B + r * lda, bytes);
+        // the first resident wave's first two rows per row group (A and B are never
+        // written by this kernel), up to 16 KiB of each, into L2 while the previous
+        // kernel drains (common.cuh).  Later waves start beside running blocks, not
+        // after a predecessor: nothing to hide there.  Same-box A/B
+        // (profiles/r02_pdl_prefetch_depth_ab.txt): GEMV 4096^2 10.5 us with one row,
+        // 9.9 with two, 10.1 with four (GESUMMV 4096^2 +1 us); 64 KiB of one row no
+        // better than 16 KiB.
+#ifndef LIFT_GEMV_PF_BYTES
+#define LIFT_GEMV_PF_BYTES 16384
+#endif
+#ifndef LIFT_GEMV_PF_ROWS
+#define LIFT_GEMV_PF_ROWS 2
+#endif
+        if ((int)blockIdx.x < pf_blocks && wr == 0 && lane < LIFT_GEMV_PF_ROWS && n > 0) {
+            const int64_t r = (int64_t)blockIdx.x * RG + g + (int64_t)lane * gridDim.x * RG;
+            const uint32_t bytes = (uint32_t)(n * 4 < LIFT_GEMV_PF_BYTES ? n * 4 : LIFT_GEMV_PF_BYTES);
+            if (r < m) {
+                bulk_prefetch_l2(A + r * lda, bytes);
+                if constexpr (NMAT == 2) bulk_prefetch_l2(B + r * lda, bytes);
+            }
         }
     }
     pdl_wait();
