@@ -652,13 +652,12 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         for (int i = 0; i < nst; ++i) mbar_init(full + i, 1);
         fence_mbar_init();
 #if LIFT_PDL_PREFETCH
-        // the ring's first stages into L2 while the previous kernel drains (common.cuh);
-        // twice or four times the ring is slower (4096^2 15.5 -> 17.4 / 19.1 us,
-        // profiles/r02_pdl_prefetch_depth_ab.txt)
-#ifndef LIFT_ATAX_PF_MULT
-#define LIFT_ATAX_PF_MULT 1
-#endif
-        for (int i = 0; i < LIFT_ATAX_PF_MULT * nst && i < nstages; ++i)
+        // the ring's first stages into L2 while the previous kernel drains (common.cuh):
+        // the whole ring when the block streams many stages, two when it streams few
+        // (profiles/r02_pdl_prefetch_depth_ab.txt: 8192^2 42.95 us with the ring vs 43.4
+        // with two, 4096^2 15.3 vs 15.1, 2048^2 10.0 vs 9.1; twice the ring is slower)
+        const int pf = nstages <= 4 * nst ? 2 : nst;
+        for (int i = 0; i < pf && i < nstages; ++i)
             bulk_prefetch_l2(A + stage_row(i) * n, (uint32_t)((int64_t)stage_rows(i) * n * 4));
 #endif
     }
