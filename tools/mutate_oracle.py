@@ -66,6 +66,26 @@ MUTATIONS = [
      "if (mag) mag[o] = 100.0 * (fabs(al) * a + fabs(be * (double)y_in[o]));", 0),
     ("sgemv_colmajor_index", "A[i + j * lda]", "A[j + i * lda]", 0),
     ("sgemv_beta_as_alpha", "y[o] = al * s + be * (double)y_in[o];", "y[o] = al * s + al * (double)y_in[o];", 0),
+    # round 2, second batch: more slips of the same kinds
+    # GESUMMV: B's products dropped from the sum, mag inflated
+    ("gesummv_dropped_B", "sb = sb + pb;", "sb = sb + 0.0 * pb;", 0),
+    ("gesummv_mag_x100", "mag[i] = fabs(al) * ma + fabs(be) * mb;", "mag[i] = 100.0 * (fabs(al) * ma + fabs(be) * mb);", 0),
+    # ATAX: mag inflated, pass 2 skips the last row, pass 2 uses x instead of t
+    ("atax_mag_x100", "if (mag) mag[j] = mag[j] + fabs((double)Ai[j]) * tmi;",
+     "if (mag) mag[j] = mag[j] + 100.0 * fabs((double)Ai[j]) * tmi;", 0),
+    ("atax_pass2_skips_last_row", "for (int64_t i = 0; i < m; ++i) {\n            const float *Ai = A + i * n;\n            const double ti",
+     "for (int64_t i = 0; i < m - 1; ++i) {\n            const float *Ai = A + i * n;\n            const double ti", 0),
+    ("atax_pass2_x_for_t", "const double ti = t[i], tmi = tm[i];", "const double ti = (double)x[i % n], tmi = tm[i];", 0),
+    # Listing 1: one tree level short, the multi-stage loop stops one stage early
+    ("listing1_tree_one_level_short", "for (int iter = 0; iter < 6; ++iter) {", "for (int iter = 0; iter < 5; ++iter) {", 0),
+    ("listing1_multistage_stops_early", "while (len > 1) {", "while (len > 128) {", 0),
+    # SGEMV: the transpose flag ignored, lda replaced by n, beta == 0 branch reads y_in
+    ("sgemv_trans_ignored", "const int64_t i = trans ? k : o, j = trans ? o : k;", "const int64_t i = o, j = k;", 0),
+    ("sgemv_lda_as_n", "A[i * lda + j]", "A[i * n + j]", 0),
+    ("sgemv_beta0_reads_y", "y[o] = al * s;", "y[o] = al * s + (double)y_in[o];", 0),
+    # partialDot: the last chunk dropped
+    ("partial_dot_last_chunk_dropped", "for (int64_t k = 0; k < groups; ++k) {\n        double s = 0.0, a = 0.0;",
+     "for (int64_t k = 0; k < groups - 1; ++k) {\n        double s = 0.0, a = 0.0;", 0),
 ]
 
 
