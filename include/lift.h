@@ -25,7 +25,11 @@
  *    with programmatic stream serialisation
  *    (PDL): they may be scheduled while the previous kernel on the stream
  *    drains, but each waits for it (griddepcontrol.wait) before touching
- *    memory, so stream order is unchanged.  LIFT_PDL=0 in the environment
+ *    memory, so stream order is unchanged.  Before that wait a kernel may
+ *    issue L2 prefetches (cp.async.bulk.prefetch.L2) of the first bytes of
+ *    its read-only inputs; a prefetch delivers no data to the program and L2
+ *    is the point of coherence, so an input the previous kernel is still
+ *    writing is read only after the wait.  LIFT_PDL=0 in the environment
  *    turns it off.  Waits inside a kernel (grid barriers) are bounded by
  *    LIFT_SPIN_TIMEOUT_MS (default 20000) and trap when exceeded.
  *  - restrict: outputs must not overlap inputs or the workspace (Fig. 7
