@@ -135,7 +135,7 @@ class ClockSampler:
                0x80: "hw_power_brake_slowdown", 0x100: "display_clock_setting"}
 
     def __init__(self, device_index: int, period_s: float = 0.005):
-        self.samples, self.reasons, self.max_mhz = [], 0, None
+        self.samples, self.mem_samples, self.reasons, self.max_mhz = [], [], 0, None
         self._stop = threading.Event()
         self.ok = False
         try:
@@ -156,6 +156,7 @@ class ClockSampler:
         while not self._stop.is_set():
             try:
                 self.samples.append(nv.nvmlDeviceGetClockInfo(self._h, nv.NVML_CLOCK_SM))
+                self.mem_samples.append(nv.nvmlDeviceGetClockInfo(self._h, nv.NVML_CLOCK_MEM))
                 self.reasons |= nv.nvmlDeviceGetCurrentClocksEventReasons(self._h)
             except Exception:
                 pass
@@ -190,6 +191,7 @@ class ClockSampler:
             return {"sm_mhz": None, "sm_max_mhz": None, "reasons": [], "note": "NVML unavailable"}
         names = [v for k, v in self.REASONS.items() if self.reasons & k and v != "gpu_idle"]
         return {"sm_mhz": statistics.median(self.samples) if self.samples else None, "sm_max_mhz": self.max_mhz,
+                "mem_mhz": statistics.median(self.mem_samples) if getattr(self, "mem_samples", None) else None,
                 "reasons": names, "samples": len(self.samples)}
 
 
@@ -640,6 +642,8 @@ def run_ours(args) -> None:
     op_ms = []
     op_min_ms = {}
     reps = 10
+    ops_sampler = ClockSampler(torch.cuda.current_device())  # the small ops move with the SM clock
+    ops_sampler.__enter__()
     l2 = torch.cuda.get_device_properties(dev).L2_cache_size
     for i, (name, op, shp, _) in enumerate(WORKLOAD):
         if i == dom:
@@ -690,6 +694,7 @@ def run_ours(args) -> None:
             ms = float(t[0])
         op_ms.append(ms)
 
+    ops_sampler.__exit__()
     ms_per_step = elapsed_ms / args.steps
     atax_algo = "fused"
     step_bytes = sum(alg_bytes(op, shp, atax_algo) for _, op, shp, _ in WORKLOAD)
@@ -757,8 +762,11 @@ def run_ours(args) -> None:
 
     # the paper's small / large sizes and configs[0]'s dot (N = 1; after the timed region)
     table1 = None
+    table1_clocks = None
     if not distributed and not args.no_table1 and args.scale == 1.0:
         table1 = {}
+        t1_sampler = ClockSampler(torch.cuda.current_device())
+        t1_sampler.__enter__()
         pool = bufs["gemv_65536x32768"]["A"].view(-1)
         tcalls = table1_calls(lift, pool, bufs["dot_2^31"]["x"], bufs["dot_2^31"]["y"], dev, l2)
         for tname, op, shp, algo, calls in tcalls:
@@ -792,6 +800,8 @@ def run_ours(args) -> None:
             if op == "atax" and algo == "fused":  # launch shape: the wide kernel's depends on the part's GPCs
                 table1[tname]["grid_blocks"], table1[tname]["cluster"] = lift.lift_atax_fused_grid(shp["m"], shp["n"])
             del g_
+        t1_sampler.__exit__()
+        table1_clocks = t1_sampler.summary()
 
     kernels_per_step = sum({"dot": 1, "gemv": 1, "gesummv": 1, "atax": 1}[op] for _, op, _, _ in WORKLOAD)
     gpu_launches = kernels_per_step * args.steps
@@ -827,7 +837,7 @@ def run_ours(args) -> None:
                                  v["frac_of_spec_peak_per_gpu"], "ncu_dram_pct_of_peak": v["ncu_dram_pct_of_peak"]}
                                 for k, v in ops.items()), key=lambda d: d["frac_of_spec_peak_per_gpu"]),
             "clocks": dict(sampler.summary(), **({"remeasured_after": first_attempt} if first_attempt else {})),
-            "ops": ops, "table1": table1,
+            "ops": ops, "ops_clocks": ops_sampler.summary(), "table1": table1, "table1_clocks": table1_clocks,
             "table1_method": "the paper's small/large sizes (Table 1) and configs[0]: >= 20 back-to-back calls "
                              "in one CUDA graph after the timed region, operands rotated over slices totalling "
                              "> 2x L2; us = median of 5 replays, us_min their minimum; ncu_* from "

@@ -669,6 +669,13 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
     // (profiles/r02_atax_pdl_trigger_ab.txt)
     pdl_wait();
     LIFT_STAMP(0);
+#ifdef LIFT_TRACE
+    if (tid == 0) {  // which SM ran this block (slot 15: a value, not a time)
+        unsigned int smid;
+        asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+        g_trace[blockIdx.x * kTraceSlots + 15] = smid;
+    }
+#endif
     if (tid == 0)  // prologue: fill the ring
         for (int i = 0; i < nst && i < nstages; ++i) issue_stage(i, i);
     // fused (all-)reduce: this call's epoch (its parity buffer is free: the previous
