@@ -641,7 +641,7 @@ def run_ours(args) -> None:
     # (operands smaller than 2x L2 are rotated over copies so every call streams from HBM)
     op_ms = []
     op_min_ms = {}
-    reps = 10
+    op_reps = {}
     ops_sampler = ClockSampler(torch.cuda.current_device())  # the small ops move with the SM clock
     ops_sampler.__enter__()
     l2 = torch.cuda.get_device_properties(dev).L2_cache_size
@@ -650,6 +650,9 @@ def run_ours(args) -> None:
             op_ms.append(dom_ms)
             continue
         by = alg_bytes(op, shp) / world
+        # enough back-to-back calls for ~2 GiB per replay (10..50): the first call of a
+        # replay has no predecessor to overlap its start with (GEMV 4096^2: 32 calls)
+        reps = op_reps[name] = min(50, max(10, -(-(1 << 31) // int(max(by, 1)))))
         copies = min(8, max(1, int(-(-2 * l2 // max(by, 1)))))
         orig = bufs[name]
         sets = [orig] + [{k: (v.clone() if k in ("A", "B", "x", "y") and op == "dot" or k in ("A", "B") else v)
@@ -770,7 +773,7 @@ def run_ours(args) -> None:
         pool = bufs["gemv_65536x32768"]["A"].view(-1)
         tcalls = table1_calls(lift, pool, bufs["dot_2^31"]["x"], bufs["dot_2^31"]["y"], dev, l2)
         for tname, op, shp, algo, calls in tcalls:
-            reps = max(20, len(calls))
+            reps = max(len(calls), min(50, max(20, -(-(1 << 31) // int(alg_bytes(op, shp, algo))))))
             seq = [calls[j % len(calls)] for j in range(reps)]
             with torch.cuda.stream(run_stream):
                 g_ = torch.cuda.CUDAGraph()
@@ -838,14 +841,15 @@ def run_ours(args) -> None:
                                 for k, v in ops.items()), key=lambda d: d["frac_of_spec_peak_per_gpu"]),
             "clocks": dict(sampler.summary(), **({"remeasured_after": first_attempt} if first_attempt else {})),
             "ops": ops, "ops_clocks": ops_sampler.summary(), "table1": table1, "table1_clocks": table1_clocks,
-            "table1_method": "the paper's small/large sizes (Table 1) and configs[0]: >= 20 back-to-back calls "
+            "table1_method": "the paper's small/large sizes (Table 1) and configs[0]: 20-50 back-to-back calls (~2 GiB) "
                              "in one CUDA graph after the timed region, operands rotated over slices totalling "
                              "> 2x L2; us = median of 5 replays, us_min their minimum; ncu_* from "
                              "profiles/table1_ncu.json (tools/table1.py under ncu)",
-            "ops_method": "dominant op: events inside the timed steps; others: 10 back-to-back calls after the "
+            "ops_method": "dominant op: events inside the timed steps; others: back-to-back calls after the "
                           "timed region" + (" (one CUDA graph)" if use_graph else "") +
-                          ", operands rotated over copies totalling > 2x L2; ms = median of 5 such runs, "
-                          "ms_min their minimum",
+                          " — enough for ~2 GiB per run, 10 to 50 (`ops_reps`) — operands rotated over copies "
+                          "totalling > 2x L2; ms = median of 5 such runs, ms_min their minimum",
+            "ops_reps": op_reps,
         }
         print(json.dumps(line), flush=True)
     if distributed:
