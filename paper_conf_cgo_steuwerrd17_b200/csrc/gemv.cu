@@ -82,18 +82,19 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
     const int g = warp / WPR;   // row group inside the block
     const int wr = warp % WPR;  // warp rank inside the row group
     if constexpr (VEC == 4 && LIFT_PDL_PREFETCH) {
-        // the first resident wave's first two rows per row group (A and B are never
-        // written by this kernel), up to 16 KiB of each, into L2 while the previous
-        // kernel drains (common.cuh).  Later waves start beside running blocks, not
-        // after a predecessor: nothing to hide there.  Same-box A/B
-        // (profiles/r02_pdl_prefetch_depth_ab.txt): GEMV 4096^2 10.5 us with one row,
-        // 9.9 with two, 10.1 with four (GESUMMV 4096^2 +1 us); 64 KiB of one row no
-        // better than 16 KiB.
+        // the first resident wave's first row per row group (A and B are never written
+        // by this kernel), up to 16 KiB of it, into L2 while the previous kernel drains
+        // (common.cuh).  Later waves start beside running blocks, not after a
+        // predecessor: nothing to hide there.  Same-box A/B: back to back, GEMV 4096^2
+        // 10.5 us with one row, 9.9 with two, 10.1 with four, 64 KiB of one row no
+        // better than 16 KiB (profiles/r02_pdl_prefetch_depth_ab.txt); launched alone
+        // (no predecessor, ncu) one row is free and two cost 0.8 us
+        // (profiles/r02_pdl_prefetch_isolated_ncu.txt): one row.
 #ifndef LIFT_GEMV_PF_BYTES
 #define LIFT_GEMV_PF_BYTES 16384
 #endif
 #ifndef LIFT_GEMV_PF_ROWS
-#define LIFT_GEMV_PF_ROWS 2
+#define LIFT_GEMV_PF_ROWS 1
 #endif
         if ((int)blockIdx.x < pf_blocks && wr == 0 && lane < LIFT_GEMV_PF_ROWS && n > 0) {
             const int64_t r = (int64_t)blockIdx.x * RG + g + (int64_t)lane * gridDim.x * RG;
