@@ -96,12 +96,21 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
 #ifndef LIFT_GEMV_PF_ROWS
 #define LIFT_GEMV_PF_ROWS 1
 #endif
+#ifndef LIFT_GESUMMV_PF_BYTES
+#define LIFT_GESUMMV_PF_BYTES LIFT_GEMV_PF_BYTES
+#endif
+// GESUMMV prefetches A's row only: back to back 4096^2 19.9 us vs 20.2 with A and B,
+// 20.8 with none; launched alone all within noise (profiles/r02_gesummv_prefetch_ab.txt)
+#ifndef LIFT_GESUMMV_PF_B
+#define LIFT_GESUMMV_PF_B 0
+#endif
         if ((int)blockIdx.x < pf_blocks && wr == 0 && lane < LIFT_GEMV_PF_ROWS && n > 0) {
             const int64_t r = (int64_t)blockIdx.x * RG + g + (int64_t)lane * gridDim.x * RG;
-            const uint32_t bytes = (uint32_t)(n * 4 < LIFT_GEMV_PF_BYTES ? n * 4 : LIFT_GEMV_PF_BYTES);
-            if (r < m) {
+            constexpr int64_t cap = NMAT == 2 ? LIFT_GESUMMV_PF_BYTES : LIFT_GEMV_PF_BYTES;
+            const uint32_t bytes = (uint32_t)(n * 4 < cap ? n * 4 : cap);
+            if (r < m && bytes > 0) {
                 bulk_prefetch_l2(A + r * lda, bytes);
-                if constexpr (NMAT == 2) bulk_prefetch_l2(B + r * lda, bytes);
+                if constexpr (NMAT == 2 && LIFT_GESUMMV_PF_B) bulk_prefetch_l2(B + r * lda, bytes);
             }
         }
     }
