@@ -493,12 +493,6 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
         }
 #endif
 #endif
-        if (discard) {    // its lines (2 per row) of every partial row are dead now
-            const int64_t e = cb + CW < c1 ? cb + CW : c1;
-            const int nl = (int)((e - cb + 7) / 8);
-            for (int k = tid; k < S * nl; k += kFusedThreads)
-                discard_l2_line(P4 + (int64_t)(k / nl) * nv + cb + 8 * (k % nl));
-        }
         if (tid < CW && c < c1) {
             float comp[4][SPL];
 #pragma unroll
@@ -511,6 +505,14 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
             }
             reinterpret_cast<float4 *>(y)[c] = make_float4(pair_tree<SPL>(comp[0]), pair_tree<SPL>(comp[1]),
                                                            pair_tree<SPL>(comp[2]), pair_tree<SPL>(comp[3]));
+        }
+        // its lines (2 per row) of every partial row are dead now; discarded after the
+        // output store is issued (-0.07 us at 4096^2, profiles/r02_atax_discard_order_ab.txt)
+        if (discard) {
+            const int64_t e = cb + CW < c1 ? cb + CW : c1;
+            const int nl = (int)((e - cb + 7) / 8);
+            for (int k = tid; k < S * nl; k += kFusedThreads)
+                discard_l2_line(P4 + (int64_t)(k / nl) * nv + cb + 8 * (k % nl));
         }
         __syncthreads();
     }
