@@ -493,18 +493,18 @@ __device__ __forceinline__ void colsum_slice(int S, int64_t nv, const float *__r
         }
 #endif
 #endif
-        if (tid < CW && c < c1) {
-            float comp[4][SPL];
+        // one thread per (column, component) runs the pairwise tree over the 32 split
+        // sums (4x shorter chains than one thread per float4 column: 16384x8192 -0.25 us,
+        // 8192x32768 -0.35, profiles/r02_atax_colsum_tree64_ab.txt); same pairs, same bits
+        if (tid < 4 * CW) {
+            const int tc = tid >> 2, comp = tid & 3;
+            if (cb + tc < c1) {
+                const float *pf = reinterpret_cast<const float *>(part);
+                float v[SPL];
 #pragma unroll
-            for (int k = 0; k < SPL; ++k) {
-                const float4 v = part[k * CW + tid];
-                comp[0][k] = v.x;
-                comp[1][k] = v.y;
-                comp[2][k] = v.z;
-                comp[3][k] = v.w;
+                for (int k = 0; k < SPL; ++k) v[k] = pf[(k * CW + tc) * 4 + comp];
+                y[4 * (cb + tc) + comp] = pair_tree<SPL>(v);
             }
-            reinterpret_cast<float4 *>(y)[c] = make_float4(pair_tree<SPL>(comp[0]), pair_tree<SPL>(comp[1]),
-                                                           pair_tree<SPL>(comp[2]), pair_tree<SPL>(comp[3]));
         }
         // its lines (2 per row) of every partial row are dead now; discarded after the
         // output store is issued (-0.07 us at 4096^2, profiles/r02_atax_discard_order_ab.txt)
