@@ -27,6 +27,26 @@
 
 namespace lift {
 
+// L2 prefetch before griddepcontrol.wait (see k_gemv): rows per first-wave row group,
+// bytes per row, and whether GESUMMV also prefetches B (-D overrides for A/B builds)
+#ifndef LIFT_GEMV_PF_BYTES
+#define LIFT_GEMV_PF_BYTES 16384
+#endif
+#ifndef LIFT_GEMV_PF_ROWS
+#define LIFT_GEMV_PF_ROWS 1
+#endif
+#ifndef LIFT_GESUMMV_PF_BYTES
+#define LIFT_GESUMMV_PF_BYTES LIFT_GEMV_PF_BYTES
+#endif
+// GESUMMV prefetches A's row only: back to back 4096^2 19.9 us vs 20.2 with A and B,
+// 20.8 with none; launched alone all within noise (profiles/r02_gesummv_prefetch_ab.txt)
+#ifndef LIFT_GESUMMV_PF_B
+#define LIFT_GESUMMV_PF_B 0
+#endif
+constexpr int kPfRows = LIFT_GEMV_PF_ROWS;
+constexpr int64_t kPfBytes = LIFT_GEMV_PF_BYTES, kPfBytesGesummv = LIFT_GESUMMV_PF_BYTES;
+constexpr bool kPfGesummvB = LIFT_GESUMMV_PF_B != 0;
+
 constexpr int kSlices = 8;
 constexpr int kVLanes = kSlices * kWarp;  // 256 virtual lanes per row
 
@@ -90,27 +110,13 @@ __global__ void __launch_bounds__(RG *WPR *kWarp) k_gemv(int64_t m, int64_t n, i
         // better than 16 KiB (profiles/r02_pdl_prefetch_depth_ab.txt); launched alone
         // (no predecessor, ncu) one row is free and two cost 0.8 us
         // (profiles/r02_pdl_prefetch_isolated_ncu.txt): one row.
-#ifndef LIFT_GEMV_PF_BYTES
-#define LIFT_GEMV_PF_BYTES 16384
-#endif
-#ifndef LIFT_GEMV_PF_ROWS
-#define LIFT_GEMV_PF_ROWS 1
-#endif
-#ifndef LIFT_GESUMMV_PF_BYTES
-#define LIFT_GESUMMV_PF_BYTES LIFT_GEMV_PF_BYTES
-#endif
-// GESUMMV prefetches A's row only: back to back 4096^2 19.9 us vs 20.2 with A and B,
-// 20.8 with none; launched alone all within noise (profiles/r02_gesummv_prefetch_ab.txt)
-#ifndef LIFT_GESUMMV_PF_B
-#define LIFT_GESUMMV_PF_B 0
-#endif
-        if ((int)blockIdx.x < pf_blocks && wr == 0 && lane < LIFT_GEMV_PF_ROWS && n > 0) {
+        if ((int)blockIdx.x < pf_blocks && wr == 0 && lane < kPfRows && n > 0) {
             const int64_t r = (int64_t)blockIdx.x * RG + g + (int64_t)lane * gridDim.x * RG;
-            constexpr int64_t cap = NMAT == 2 ? LIFT_GESUMMV_PF_BYTES : LIFT_GEMV_PF_BYTES;
+            constexpr int64_t cap = NMAT == 2 ? kPfBytesGesummv : kPfBytes;
             const uint32_t bytes = (uint32_t)(n * 4 < cap ? n * 4 : cap);
             if (r < m && bytes > 0) {
                 bulk_prefetch_l2(A + r * lda, bytes);
-                if constexpr (NMAT == 2 && LIFT_GESUMMV_PF_B) bulk_prefetch_l2(B + r * lda, bytes);
+                if constexpr (NMAT == 2 && kPfGesummvB) bulk_prefetch_l2(B + r * lda, bytes);
             }
         }
     }
