@@ -764,6 +764,11 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
             const float *pb = red + (buf ^ 1) * CR * kFusedWarps;
             float t[CR];  // t_r = A_r . x: the pairwise tree over the 16 warp sums
             warp_trees<CR>(pb, lane, t);
+#ifdef LIFT_EXP_GEMV_RING  // experiment (tools only): the ring as a GEMV, t_r written out
+            if (tid == 0)
+                for (int i = 0; i < CR; ++i)
+                    if (i < prow) y[stage_row(k - 1) + i] = t[i];
+#else
 #pragma unroll
             for (int i = 0; i < CR; ++i) {
                 if (i < prow) {
@@ -771,6 +776,7 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
                     for (int q = 0; q < QC; ++q) fma4s(yr[q], prev[i][q], t[i]);
                 }
             }
+#endif
         }
         if (rows == 0) return true;
         prow = rows;
@@ -788,6 +794,9 @@ __global__ void __launch_bounds__(kFusedThreads, 1)
         if (step(rb2, ra)) break;
     }
     LIFT_STAMP(3);
+#ifdef LIFT_EXP_GEMV_RING
+    return;
+#endif
     float4 *P4 = reinterpret_cast<float4 *>(P) + (int64_t)blockIdx.x * nv;
 #pragma unroll
     for (int q = 0; q < QC; ++q) {
